@@ -1,0 +1,451 @@
+#!/usr/bin/env python3
+"""bench.py -- SeparableConvolution on B200: output Mpixels/s and HBM GB/s per kernel width.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+                    [--workload image|batch] [--widths 3,5,...,17]
+
+Workload (BASELINE.json configs[3], the metric's configuration): one 16384 x 16384
+float32 image, kernel widths K = 3, 5, ..., 17.  A "step" is one SeparableConvolution
+of the image per width (8 passes of the whole hot path), each with the tuned AUTO
+variant.  At N > 1 (torchrun) the image is split into N row bands, one per GPU, and
+every pass exchanges the (K-1)-row halo with NCCL send/recv inside the C ABI
+(sepconv_run_band); scaling is strong (fixed image).  --workload batch is
+configs[4] (64 x 4096^2, K = 11, images sharded over ranks, no exchange).
+
+value = output pixels of the whole job per step / max-over-ranks device time
+(CUDA events, inputs resident in HBM; the 1.07 GB image is larger than the 126 MB
+L2, so no flush is needed between steps).  e2e = the same metric through
+sepconv_run_host with pinned HOST buffers, copies inside the timed region.
+The oracle (oracle/, test infrastructure) runs only in the cpu_baseline leg and in
+--impl reference, on a bounded sample, on rank 0.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import tempfile
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+from paper_conf_asplos_phothilimthanaara13_b200 import synth  # noqa: E402
+
+METRIC = "output Mpixels/s and HBM GB/s (% of B200 peak) per kernel width, 1/2/4/8 GPUs"
+HBM_FALLBACK_GBS = 6650.0          # /opt/skills/guides/B200_PROFILING.md fallback (used only if MEASURED_PEAKS.json is absent)
+NOMINAL_HBM_GBS = 8000.0           # BASELINE.json north_star "roughly 8 TB/s"
+
+
+def parse_args():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--workload", choices=["image", "batch"], default="image")
+    ap.add_argument("--widths", default="3,5,7,9,11,13,15,17")
+    ap.add_argument("--size", type=int, default=16384, help="image side (image workload)")
+    ap.add_argument("--variant", default="auto")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle time for the cpu_baseline sample")
+    ap.add_argument("--tune-reps", type=int, default=10)
+    return ap.parse_args()
+
+
+def peaks():
+    path = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(path) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs: torch D2D copy)"
+    except Exception:
+        return HBM_FALLBACK_GBS, "fallback (B200_PROFILING.md)"
+
+
+def dist_env():
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return world, rank, local
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons during the timed region (B200_PROFILING.md recipe)."""
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.file = tempfile.NamedTemporaryFile("w+", suffix=".csv", delete=False)
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.index), "--query-gpu=" + self.FIELDS,
+                                          "--format=csv,noheader,nounits", "-lms", "100"],
+                                         stdout=self.file, stderr=subprocess.DEVNULL)
+            time.sleep(0.3)
+        except Exception:
+            self.proc = None
+        return self
+
+    def __exit__(self, *exc):
+        if self.proc:
+            time.sleep(0.25)
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:
+                self.proc.kill()
+
+    def summary(self):
+        if not self.proc:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        self.file.flush()
+        rows = []
+        with open(self.file.name) as f:
+            for line in f:
+                parts = [p.strip() for p in line.split(",")]
+                if len(parts) < 9:
+                    continue
+                try:
+                    rows.append((float(parts[1]), float(parts[2]), float(parts[3]), parts[5:9]))
+                except ValueError:
+                    continue
+        os.unlink(self.file.name)
+        if not rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["no samples"]}
+        loaded = [r for r in rows if r[2] > 200] or rows
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in rows for i, v in enumerate(r[3]) if v.lower().startswith("active")})
+        return {"sm_mhz": statistics.median(r[0] for r in loaded), "sm_max_mhz": max(r[1] for r in rows),
+                "power_w_max": max(r[2] for r in rows), "samples": len(rows), "reasons": reasons}
+
+
+# --------------------------------------------------------------------------------------------
+def oracle_sample(img_rows_fn, W, widths, target_s, nthreads=0):
+    """Time the oracle (as it stands) on the first S output rows of the image for every width."""
+    import oracle
+    cores = nthreads or oracle.num_cpus()
+    kmax = max(widths)
+
+    def run(S):
+        src = img_rows_fn(S + kmax - 1)
+        t0 = time.perf_counter()
+        px = 0
+        for K in widths:
+            out = oracle.convolve2d(np.ascontiguousarray(src[:S + K - 1]), synth.binomial_kernel(K), nthreads=cores)
+            px += out.size
+        return time.perf_counter() - t0, px
+
+    t_probe, _ = run(4)
+    S = int(max(4, min(4096, 4 * target_s / max(t_probe, 1e-4))))
+    t, px = run(S)
+    return {"value": px / t / 1e6, "unit": "Mpixels/s", "cores": cores, "kind": "oracle",
+            "sample": f"first {S} output rows x {W - min(widths) + 1}..{W - kmax + 1} cols of the image, "
+                      f"widths {widths[0]}..{widths[-1]} (K^2 double MACs/px), {t:.1f} s",
+            "seconds": t, "pixels": px}
+
+
+def emit(d):
+    print(json.dumps(d), flush=True)
+
+
+# --------------------------------------------------------------------------------------------
+def run_reference(args):
+    """--impl reference: the oracle (the paper's definition in plain C, double) on host cores."""
+    world, rank, _ = dist_env()
+    if rank != 0:
+        return 0
+    widths = [int(x) for x in args.widths.split(",")] if args.workload == "image" else [11]
+    W = args.size if args.workload == "image" else 4096
+    H = W
+    seed = synth.BENCH_SEED_BASE + (3 if args.workload == "image" else 4)
+    per_step_s = max(2.0, 60.0 / max(1, args.steps + args.warmup))
+    rows_cache = {}
+
+    def img_rows(n):
+        if n not in rows_cache:
+            rows_cache[n] = synth.uniform_image(H, W, seed, rows=(0, min(H, n)))
+        return rows_cache[n]
+
+    for _ in range(args.warmup):
+        oracle_sample(img_rows, W, widths, per_step_s / 4)
+    vals, times = [], []
+    last = None
+    for _ in range(args.steps):
+        last = oracle_sample(img_rows, W, widths, per_step_s)
+        vals.append(last["value"])
+        times.append(last["seconds"])
+    value = statistics.median(vals)
+    cfg = {"workload": "16384x16384 float32 image, widths 3..17 odd" if args.workload == "image"
+           else "64 x 4096x4096 float32, width 11", "widths": widths, "sample": last["sample"]}
+    emit({"impl": "reference", "metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world,
+          "steps": args.steps, "warmup": args.warmup, "ms_per_step": statistics.median(times) * 1e3,
+          "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
+          "data": "synthetic", "config": cfg,
+          "cpu_baseline": {"value": value, "unit": "Mpixels/s", "cores": last["cores"], "kind": "oracle",
+                           "sample": last["sample"]},
+          "e2e": {"value": value, "unit": "Mpixels/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}})
+    return 0
+
+
+# --------------------------------------------------------------------------------------------
+def main():
+    args = parse_args()
+    if args.impl == "reference":
+        return run_reference(args)
+
+    import torch
+    from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+
+    world, rank, local = dist_env()
+    if world != args.gpus:
+        print(f"[bench] warning: --gpus {args.gpus} but WORLD_SIZE={world}; using WORLD_SIZE", file=sys.stderr)
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    dist = None
+    if world > 1:
+        import torch.distributed as dist
+        dist.init_process_group("nccl", device_id=dev)
+
+    peak_gbs, peak_src = peaks()
+    widths = [int(x) for x in args.widths.split(",")]
+    if args.workload == "batch":
+        widths = [11]
+        N_img, H = 64, 4096
+        W = H
+    else:
+        N_img, H = 1, args.size
+        W = H
+    seed = synth.BENCH_SEED_BASE + (3 if args.workload == "image" else 4)
+    stream = torch.cuda.current_stream(dev)
+
+    # ---- this rank's share of the input, resident in HBM ----
+    if args.workload == "image":
+        bands = {K: sc.band(H, K, world, rank) for K in widths}
+        kmax = max(widths)
+        # one buffer holding the union of the bands' rows (bands shift slightly with K)
+        r_lo = min(b[0] for b in bands.values())
+        r_hi = max(b[0] + b[3] for b in bands.values())
+        host_img = synth.uniform_image(H, W, seed, rows=(r_lo, min(H, r_hi)))
+        dev_img = torch.empty((r_hi - r_lo + kmax, W), dtype=torch.float32, device=dev)
+        dev_img[:host_img.shape[0]].copy_(torch.from_numpy(host_img))
+        plans, outs, ins = {}, {}, {}
+        for K in widths:
+            r0, rows, owned, alloc = bands[K]
+            p = sc.Plan(alloc, W, K)
+            if world > 1:
+                uid = sc.nccl_unique_id() if rank == 0 else bytes(sc.NCCL_ID_BYTES)
+                t = torch.tensor(list(uid), dtype=torch.uint8, device=dev)
+                dist.broadcast(t, 0)
+                p.comm_init(bytes(t.cpu().tolist()), world, rank)
+            plans[K] = p
+            outs[K] = torch.empty((rows, W - K + 1), dtype=torch.float32, device=dev)
+            # the band's own input rows; rows past `owned` are the halo, written by run_band
+            ins[K] = dev_img[r0 - r_lo:r0 - r_lo + alloc]
+            if world > 1:
+                ins[K] = ins[K].clone()     # run_band writes the halo rows: keep bands private per width
+        out_px_rank = {K: outs[K].numel() for K in widths}
+        out_px_job = {K: (H - K + 1) * (W - K + 1) for K in widths}
+        in_rows_job = {K: H for K in widths}
+    else:
+        per = N_img // world
+        n0 = rank * per
+        host_img = np.stack([synth.uniform_image(H, W, seed, n=n0 + i) for i in range(per)])
+        dev_img = torch.from_numpy(host_img).to(dev)
+        K = widths[0]
+        plans = {K: sc.Plan(H, W, K, n=per)}
+        outs = {K: torch.empty((per, H - K + 1, W - K + 1), dtype=torch.float32, device=dev)}
+        ins = {K: dev_img}
+        out_px_rank = {K: outs[K].numel()}
+        out_px_job = {K: N_img * (H - K + 1) * (W - K + 1)}
+        in_rows_job = {K: N_img * H}
+
+    kernels = {K: synth.binomial_kernel(K) for K in widths}
+
+    # ---- tune (the paper's install-time autotuning): per width, per rank ----
+    choices = {}
+    for K in widths:
+        choices[K] = plans[K].tune(reps=args.tune_reps)
+    torch.cuda.synchronize()
+
+    def one_pass(K):
+        if world > 1 and args.workload == "image":
+            plans[K].run_band(ins[K], kernels[K], outs[K], args.variant, stream)
+        else:
+            plans[K].run(ins[K], kernels[K], outs[K], args.variant, stream)
+
+    # ---- warm-up ----
+    for _ in range(max(args.warmup, 0)):
+        for K in widths:
+            one_pass(K)
+    torch.cuda.synchronize()
+    if dist:
+        dist.barrier()
+
+    # ---- timed region: CUDA events on the launching stream, per pass and per step ----
+    ev = {K: [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+              for _ in range(args.steps)] for K in widths}
+    e_start, e_end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    launches0 = sc.launch_count()
+    with ClockSampler(local) as clk:
+        torch.cuda.synchronize()
+        if dist:
+            dist.barrier()
+        e_start.record(stream)
+        for s in range(args.steps):
+            for K in widths:
+                ev[K][s][0].record(stream)
+                one_pass(K)
+                ev[K][s][1].record(stream)
+        e_end.record(stream)
+        torch.cuda.synchronize()
+        if dist:
+            dist.barrier()
+    launches = sc.launch_count() - launches0
+    total_ms = e_start.elapsed_time(e_end)
+    per_k_ms = {K: sum(a.elapsed_time(b) for a, b in ev[K]) / args.steps for K in widths}
+    if dist:
+        t = torch.tensor([total_ms] + [per_k_ms[K] for K in widths], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        total_ms = float(t[0])
+        per_k_ms = {K: float(t[1 + i]) for i, K in enumerate(widths)}
+    ms_per_step = total_ms / args.steps
+    px_step = sum(out_px_job.values())
+    value = px_step / (ms_per_step * 1e-3) / 1e6
+
+    # algorithmic bytes: read every input once, write every output once, + received halo
+    def alg_bytes(K):
+        b = 4 * (in_rows_job[K] * W + out_px_job[K])
+        if world > 1 and args.workload == "image":
+            b += 4 * (K - 1) * W * (world - 1)
+        return b
+
+    per_width = {}
+    for K in widths:
+        t_s = per_k_ms[K] * 1e-3
+        gbs = alg_bytes(K) / t_s / 1e9
+        per_width[str(K)] = {"variant": sc.Choice(*[getattr(choices[K], f) for f in
+                                                     ("algo", "mapping", "fused")]).name,
+                             "us": per_k_ms[K] * 1e3, "mpix_s": out_px_job[K] / t_s / 1e6, "gbs": gbs,
+                             "frac_of_measured": gbs / (peak_gbs * world),
+                             "frac_of_8tbs": gbs / (NOMINAL_HBM_GBS * world)}
+
+    # roofline for the dominant kernel family (the AUTO choice of most widths)
+    names = [per_width[str(K)]["variant"] for K in widths]
+    dom = max(set(names), key=lambda n: sum(per_k_ms[K] for K in widths if per_width[str(K)]["variant"] == n))
+    dom_k = [K for K in widths if per_width[str(K)]["variant"] == dom]
+    dom_bytes = sum(alg_bytes(K) for K in dom_k) / world          # per GPU, per launch set
+    dom_s = sum(per_k_ms[K] for K in dom_k) * 1e-3
+    achieved = dom_bytes / dom_s / 1e9
+    traffic = None
+    tr_path = os.path.join(ROOT, "profiles", "traffic.json")
+    if os.path.exists(tr_path):
+        try:
+            tr = json.load(open(tr_path))
+            vals = [tr[f"{dom}:K{K}"] for K in dom_k if f"{dom}:K{K}" in tr and args.workload == "image"
+                    and world == 1 and H == 16384]
+            if len(vals) == len(dom_k):
+                traffic = sum(vals) / len(vals)
+        except Exception:
+            traffic = None
+    roofline = {"bound": "hbm", "kernel": dom, "widths": dom_k, "achieved": achieved, "peak": peak_gbs,
+                "unit": "GB/s", "frac": achieved / peak_gbs, "traffic": traffic, "peak_source": peak_src,
+                "algorithmic_bytes_per_launch": dom_bytes / len(dom_k),
+                "frac_of_8tbs": achieved / NOMINAL_HBM_GBS}
+
+    # ---- e2e: the public API with pinned HOST buffers, copies inside the timed region ----
+    e2e = None
+    if not args.no_e2e:
+        e2e_steps = max(1, min(args.steps, 2))
+        h_out = {}
+        hplans = {}
+        if args.workload == "image":
+            bands = {K: sc.band(H, K, world, rank) for K in widths}
+            h_in = torch.from_numpy(host_img).pin_memory()
+            for K in widths:
+                r0, rows, owned, alloc = bands[K]
+                hplans[K] = sc.Plan(alloc, W, K)
+                hplans[K].tune(reps=3)
+                h_out[K] = torch.empty((rows, W - K + 1), dtype=torch.float32).pin_memory()
+        else:
+            h_in = torch.from_numpy(host_img).pin_memory()
+            K = widths[0]
+            hplans[K] = plans[K]
+            h_out[K] = torch.empty(tuple(outs[K].shape), dtype=torch.float32).pin_memory()
+        h2d = d2h = 0
+
+        def e2e_pass(K):
+            nonlocal h2d, d2h
+            if args.workload == "image":
+                r0, rows, owned, alloc = bands[K]
+                src = h_in[r0 - r_lo:r0 - r_lo + alloc]
+                hplans[K].run_host(src, kernels[K], h_out[K], args.variant, stream)
+                h2d += src.numel() * 4
+            else:
+                hplans[K].run_host(h_in, kernels[K], h_out[K], args.variant, stream)
+                h2d += h_in.numel() * 4
+            d2h += h_out[K].numel() * 4
+
+        for K in widths:
+            e2e_pass(K)
+        h2d = d2h = 0
+        torch.cuda.synchronize()
+        if dist:
+            dist.barrier()
+        t0 = time.perf_counter()
+        for _ in range(e2e_steps):
+            for K in widths:
+                e2e_pass(K)
+        torch.cuda.synchronize()
+        el = time.perf_counter() - t0
+        if dist:
+            t = torch.tensor([el, h2d, d2h], dtype=torch.float64, device=dev)
+            tmax = t.clone()
+            dist.all_reduce(tmax, op=dist.ReduceOp.MAX)
+            dist.all_reduce(t, op=dist.ReduceOp.SUM)
+            el, h2d, d2h = float(tmax[0]), float(t[1]), float(t[2])
+        e2e = {"value": px_step * e2e_steps / el / 1e6, "unit": "Mpixels/s",
+               "h2d_bytes_per_step": int(h2d / e2e_steps), "d2h_bytes_per_step": int(d2h / e2e_steps),
+               "ms_per_step": el / e2e_steps * 1e3, "api": "sepconv_run_host (pinned host buffers)"}
+
+    # ---- cpu_baseline: the oracle as it stands, bounded sample, rank 0 at N=1 only ----
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        if args.workload == "image":
+            cpu = oracle_sample(lambda n: host_img[:n], W, widths, args.cpu_seconds)
+        else:
+            cpu = oracle_sample(lambda n: host_img[0][:n], W, widths, args.cpu_seconds)
+        cpu = {k: v for k, v in cpu.items() if k not in ("seconds", "pixels")}
+
+    if rank == 0:
+        cfg = {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
+                            if args.workload == "image" else f"{N_img} x {H}x{W} float32 images, width 11"),
+               "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
+               "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
+               "l2": "inputs larger than L2 (no flush)" if (H * W * 4 * N_img) > 2 * 126e6 else "L2-resident",
+               "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
+                               else f"images sharded x{world}" if world > 1 else "1 GPU")}
+        emit({"metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world, "steps": args.steps,
+              "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "strong",
+              "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": cfg,
+              "hbm_gbs": sum(alg_bytes(K) for K in widths) / (ms_per_step * 1e-3) / 1e9,
+              "per_width": per_width, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
+              "gpu_launches": int(launches), "clocks": clk.summary()})
+    if dist:
+        dist.barrier()
+        dist.destroy_process_group()
+    return 0
+
+
+if __name__ == "__main__":
+    sys.exit(main())

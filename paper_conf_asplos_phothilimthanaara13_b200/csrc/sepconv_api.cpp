@@ -1,0 +1,532 @@
+// sepconv_api.cpp -- the C ABI of include/sepconv.h: plans, validation, variant
+// resolution and kernel launches.  Tuning is in sepconv_tune.cpp, the
+// host-resident pipeline in sepconv_host.cpp, row bands + NCCL in sepconv_band.cpp.
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <mutex>
+#include <new>
+#include <string>
+
+#include "sepconv_internal.h"
+
+namespace sepconv {
+
+std::atomic<uint64_t> g_launches{0};
+static thread_local std::string t_last_error;
+
+sepconv_status_t fail(sepconv_status_t st, const char *fmt, ...) {
+    char msg[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(msg, sizeof msg, fmt, ap);
+    va_end(ap);
+    t_last_error = msg;
+    return st;
+}
+
+sepconv_status_t cuda_fail(cudaError_t e, const char *what) {
+    return fail(e == cudaErrorMemoryAllocation ? SEPCONV_E_NOMEM : SEPCONV_E_CUDA, "%s: %s (%s)", what,
+                cudaGetErrorString(e), cudaGetErrorName(e));
+}
+
+static void clear_error() { t_last_error.clear(); }
+
+// ---- device / driver helpers ---------------------------------------------------------------
+typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *, const cuuint64_t *,
+                                  const cuuint64_t *, const cuuint32_t *, const cuuint32_t *, CUtensorMapInterleave,
+                                  CUtensorMapSwizzle, CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
+
+static EncodeTiledFn encode_fn() {
+    static EncodeTiledFn fn = nullptr;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        void *p = nullptr;
+        cudaDriverEntryPointQueryResult q;
+        if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
+            q == cudaDriverEntryPointSuccess)
+            fn = reinterpret_cast<EncodeTiledFn>(p);
+    });
+    return fn;
+}
+
+static sepconv_status_t query_device(int device, DeviceInfo *out) {
+    int count = 0;
+    cudaError_t e = cudaGetDeviceCount(&count);
+    if (e != cudaSuccess || count == 0)
+        return fail(SEPCONV_E_UNSUPPORTED, "no CUDA device (%s)", cudaGetErrorString(e));
+    if (device < 0) SC_CUDA(cudaGetDevice(&device));
+    if (device >= count) return fail(SEPCONV_E_INVALID, "device %d out of range (%d devices)", device, count);
+    cudaDeviceProp prop;
+    SC_CUDA(cudaGetDeviceProperties(&prop, device));
+    if (prop.major != 10)
+        return fail(SEPCONV_E_UNSUPPORTED, "device %d is sm_%d%d; this library is built for sm_100a (B200)", device,
+                    prop.major, prop.minor);
+    out->device = device;
+    out->sms = prop.multiProcessorCount;
+    out->major = prop.major;
+    out->minor = prop.minor;
+    out->l2 = static_cast<size_t>(prop.l2CacheSize);
+    out->smem_optin = prop.sharedMemPerBlockOptin;
+    out->name = prop.name;
+    return SEPCONV_OK;
+}
+
+struct DeviceGuard {
+    int prev = -1;
+    bool ok = true;
+    explicit DeviceGuard(int dev) {
+        cudaGetDevice(&prev);
+        if (prev != dev) ok = cudaSetDevice(dev) == cudaSuccess;
+    }
+    ~DeviceGuard() {
+        if (prev >= 0) cudaSetDevice(prev);
+    }
+};
+
+// ---- validation ---------------------------------------------------------------------------------
+sepconv_status_t check_kernel(const float *kernel, int K) {
+    if (!kernel) return fail(SEPCONV_E_INVALID, "kernel is NULL (expected a host pointer to %d floats)", K);
+    return SEPCONV_OK;
+}
+
+static bool aligned(const void *p, size_t a) { return (reinterpret_cast<uintptr_t>(p) % a) == 0; }
+
+Geometry plan_geometry(sepconv_plan_t plan) {
+    Geometry g;
+    g.K = plan->k;
+    g.nimg = static_cast<int>(plan->n);
+    g.in_rows = static_cast<int>(plan->h);
+    g.in_cols = static_cast<int>(plan->w);
+    g.ld_in = plan->ld_in;
+    g.in_img = plan->h * plan->ld_in;
+    g.out_cols = static_cast<int>(plan->wo);
+    g.ld_out = plan->ld_out;
+    g.out_img = plan->ho * plan->ld_out;
+    g.row_begin = 0;
+    g.rows = static_cast<int>(plan->ho);
+    return g;
+}
+
+static long long extent_floats(long long nimg, long long img, long long rows, long long ld, long long cols) {
+    return (nimg - 1) * img + (rows - 1) * ld + cols;
+}
+
+// ---- launching ------------------------------------------------------------------------------------
+static int map_index(bool tma, bool vec16) { return tma ? MAP_TMA : (vec16 ? MAP_DIRECT_VEC : MAP_DIRECT); }
+
+static sepconv_status_t prepare_func(const KernelInfo &ki, int dev, const DeviceInfo &di, int *blocks_per_sm) {
+    // attribute setting is cheap but not free: cache per (function, device)
+    static std::mutex mu;
+    static std::map<std::pair<const void *, int>, int> occ_cache;
+    std::lock_guard<std::mutex> lock(mu);
+    auto key = std::make_pair(ki.func, dev);
+    auto it = occ_cache.find(key);
+    if (it != occ_cache.end()) {
+        *blocks_per_sm = it->second;
+        return SEPCONV_OK;
+    }
+    if (ki.smem > di.smem_optin)
+        return fail(SEPCONV_E_UNSUPPORTED, "kernel needs %zu B shared memory, device allows %zu", ki.smem,
+                    di.smem_optin);
+    SC_CUDA(cudaFuncSetAttribute(ki.func, cudaFuncAttributeMaxDynamicSharedMemorySize, static_cast<int>(ki.smem)));
+    int occ = 0;
+    SC_CUDA(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, ki.func, ki.threads, ki.smem));
+    if (occ < 1) return fail(SEPCONV_E_UNSUPPORTED, "kernel cannot be resident (occupancy 0)");
+    occ_cache[key] = occ;
+    *blocks_per_sm = occ;
+    return SEPCONV_OK;
+}
+
+static sepconv_status_t make_tmap(sepconv_plan_t plan, CUtensorMap *map, const float *base, int cols, int rows,
+                                  int nimg, long long ld, long long img, int box_w, int box_h) {
+    EncodeTiledFn enc = encode_fn();
+    if (!enc) return fail(SEPCONV_E_CUDA, "cuTensorMapEncodeTiled unavailable from the driver");
+    const long long key2 = ((((static_cast<long long>(cols) * 1315423911LL + rows) * 2654435761LL + nimg) * 97 + ld) *
+                                31 + img) * 131 + box_w * 1024 + box_h;
+    auto key = std::make_pair(reinterpret_cast<uintptr_t>(base), key2);
+    auto it = plan->tmaps.maps.find(key);
+    if (it != plan->tmaps.maps.end()) {
+        *map = it->second;
+        return SEPCONV_OK;
+    }
+    cuuint64_t dims[3] = {static_cast<cuuint64_t>(cols), static_cast<cuuint64_t>(rows), static_cast<cuuint64_t>(nimg)};
+    cuuint64_t strides[2] = {static_cast<cuuint64_t>(ld) * 4, static_cast<cuuint64_t>(img) * 4};
+    cuuint32_t box[3] = {static_cast<cuuint32_t>(box_w), static_cast<cuuint32_t>(box_h), 1};
+    cuuint32_t estr[3] = {1, 1, 1};
+    CUresult r = enc(map, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<float *>(base), dims, strides, box, estr,
+                     CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (r != CUDA_SUCCESS) return fail(SEPCONV_E_CUDA, "cuTensorMapEncodeTiled failed (CUresult %d)", (int)r);
+    if (plan->tmaps.maps.size() > 64) plan->tmaps.maps.clear();
+    plan->tmaps.maps[key] = *map;
+    return SEPCONV_OK;
+}
+
+static bool tma_ok(const float *base, long long ld, long long img) {
+    return aligned(base, 16) && (ld % 4) == 0 && (img % 4) == 0;
+}
+
+static int grid_for(const DeviceInfo &di, int occ, long long total) {
+    long long g = static_cast<long long>(di.sms) * occ;
+    if (g > total) g = total;
+    return static_cast<int>(std::max<long long>(g, 1));
+}
+
+// One streaming pass (ROWS, COLS or SEP) over geometry g.
+static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geometry &g, const float *in,
+                                         long long ld_in, long long in_img, int in_cols, float *out,
+                                         long long ld_out, long long out_img, int out_cols, int rows_total,
+                                         const float *kernel, bool want_tma, cudaStream_t st) {
+    const int K = g.K;
+    const bool tma = want_tma && tma_ok(in, ld_in, in_img);
+    const bool vec = aligned(in, 16) && (ld_in % 4) == 0 && (in_img % 4) == 0;
+    const int map = map_index(tma, vec);
+    KernelInfo ki = op == OP_ROWS ? stream_rows_info(map, K) : op == OP_COLS ? stream_cols_info(map, K)
+                                                                            : stream_sep_info(map, K);
+    int occ = 0;
+    sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);
+    if (s != SEPCONV_OK) return s;
+
+    StreamParams p;
+    std::memset(&p, 0, sizeof p);
+    p.in = in;
+    p.out = out;
+    p.in_img_stride = in_img;
+    p.out_img_stride = out_img;
+    p.ld_in = ld_in;
+    p.ld_out = ld_out;
+    p.in_rows = g.in_rows;
+    p.in_cols = in_cols;
+    p.out_cols = out_cols;
+    p.row_begin = g.row_begin;
+    p.rows = rows_total;
+    p.nimg = g.nimg;
+    const int cta_cols = kNW * kWarpCols;
+    p.nstrips = (out_cols + cta_cols - 1) / cta_cols;
+    p.total = static_cast<long long>(g.nimg) * p.nstrips * rows_total;
+    for (int i = 0; i < K; ++i) p.k[i] = kernel[i];
+    if (tma) {
+        const bool halo = op != OP_COLS;
+        const int sr = op == OP_ROWS ? 16 : K * std::max(1, 20 / K);
+        s = make_tmap(plan, &p.tmap, in, in_cols, g.in_rows, g.nimg, ld_in, in_img, box_width(K, halo), sr);
+        if (s != SEPCONV_OK) return s;
+    }
+    if (p.total <= 0) return SEPCONV_OK;
+    const int grid = grid_for(plan->dev, occ, p.total);
+    cudaError_t e = op == OP_ROWS ? stream_rows_launch(map, K, p, grid, st)
+                    : op == OP_COLS ? stream_cols_launch(map, K, p, grid, st)
+                                    : stream_sep_launch(map, K, p, grid, st);
+    if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
+    g_launches.fetch_add(1, std::memory_order_relaxed);
+    return SEPCONV_OK;
+}
+
+static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const float *in, float *out,
+                                  const float *kernel, bool want_tma, cudaStream_t st) {
+    const int K = g.K;
+    const bool tma = want_tma && tma_ok(in, g.ld_in, g.in_img);
+    const bool vec = aligned(in, 16) && (g.ld_in % 4) == 0 && (g.in_img % 4) == 0;
+    const int map = map_index(tma, vec);
+    KernelInfo ki = conv2d_info(map, K);
+    int occ = 0;
+    sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);
+    if (s != SEPCONV_OK) return s;
+    Conv2DParams p;
+    std::memset(&p, 0, sizeof p);
+    p.in = in;
+    p.out = out;
+    p.in_img_stride = g.in_img;
+    p.out_img_stride = g.out_img;
+    p.ld_in = g.ld_in;
+    p.ld_out = g.ld_out;
+    p.in_rows = g.in_rows;
+    p.in_cols = g.in_cols;
+    p.out_cols = g.out_cols;
+    p.row_begin = g.row_begin;
+    p.rows = g.rows;
+    p.nimg = g.nimg;
+    const int cta_cols = kNW * kWarpCols;
+    p.nstrips = (g.out_cols + cta_cols - 1) / cta_cols;
+    p.total = static_cast<long long>(g.nimg) * p.nstrips * g.rows;
+    // w_ji = fl(k_i * k_j): the outer-product weights of Convolve2D, rounded once
+    for (int j = 0; j < K; ++j)
+        for (int i = 0; i < K; ++i) p.w[j * K + i] = kernel[i] * kernel[j];
+    if (tma) {
+        s = make_tmap(plan, &p.tmap, in, g.in_cols, g.in_rows, g.nimg, g.ld_in, g.in_img, box_width(K, true),
+                      Conv2DCfg<1>::SR);
+        if (s != SEPCONV_OK) return s;
+    }
+    if (p.total <= 0) return SEPCONV_OK;
+    const int grid = grid_for(plan->dev, occ, p.total);
+    cudaError_t e = conv2d_launch(map, K, p, grid, st);
+    if (e != cudaSuccess) return cuda_fail(e, "conv2d kernel launch");
+    g_launches.fetch_add(1, std::memory_order_relaxed);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t ensure_buf(sepconv_plan_t plan) {
+    if (plan->buf) return SEPCONV_OK;
+    plan->ld_buf = (plan->wo + 3) & ~3LL;
+    plan->buf_floats = static_cast<size_t>(plan->n * plan->h * plan->ld_buf);
+    cudaError_t e = cudaMalloc(&plan->buf, plan->buf_floats * sizeof(float));
+    if (e != cudaSuccess) {
+        plan->buf = nullptr;
+        return cuda_fail(e, "cudaMalloc(unfused separable buffer)");
+    }
+    return SEPCONV_OK;
+}
+
+sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const float *in, float *out,
+                                  const float *kernel, const Candidate &c, float *buf, long long ld_buf,
+                                  cudaStream_t st) {
+    const bool tma = c.mapping == SEPCONV_MAP_TMA;
+    if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st);
+    if (c.fused)
+        return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img,
+                                g.out_cols, g.rows, kernel, tma, st);
+    // Choice 2 as the paper writes it: ConvolveRows into buffer, then ConvolveColumns.
+    // The buffer holds the rows this launch's output rows need: [row_begin, row_begin + rows + K - 1).
+    if (!buf) return fail(SEPCONV_E_INVALID, "unfused separable needs a workspace");
+    const int brows = g.rows + g.K - 1;
+    Geometry gr = g;
+    gr.row_begin = 0;
+    const long long buf_img = static_cast<long long>(brows) * ld_buf;
+    // ROWS: input rows [row_begin, row_begin+brows) -> buf rows [0, brows)
+    gr.in_rows = g.in_rows;
+    {
+        Geometry gg = g;
+        gg.rows = brows;
+        // shift the input pointer so buf row 0 = input row row_begin
+        const float *in0 = in + static_cast<long long>(g.row_begin) * g.ld_in;
+        gg.in_rows = g.in_rows - g.row_begin;
+        gg.row_begin = 0;
+        sepconv_status_t s = launch_stream_op(plan, OP_ROWS, gg, in0, g.ld_in, g.in_img, g.in_cols, buf, ld_buf,
+                                              buf_img, g.out_cols, brows, kernel, tma, st);
+        if (s != SEPCONV_OK) return s;
+    }
+    {
+        Geometry gc = g;
+        gc.in_rows = brows;
+        gc.row_begin = 0;
+        float *out0 = out + static_cast<long long>(g.row_begin) * g.ld_out;
+        return launch_stream_op(plan, OP_COLS, gc, buf, ld_buf, buf_img, g.out_cols, out0, g.ld_out, g.out_img,
+                                g.out_cols, g.rows, kernel, tma, st);
+    }
+}
+
+// Static default before tuning (R16): fused separable with TMA for K >= 2
+// (one HBM pass, 2K FMA/px), 2D with TMA for K = 1.
+static Candidate default_candidate(int K, sepconv_variant_t v) {
+    if (v == SEPCONV_2D || (v == SEPCONV_AUTO && K == 1)) return {SEPCONV_2D, SEPCONV_MAP_TMA, 0};
+    return {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1};
+}
+
+Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v) {
+    const int idx = v == SEPCONV_2D ? 0 : v == SEPCONV_SEPARABLE ? 1 : 2;
+    if (plan->tuned) {
+        const sepconv_choice_t &c = plan->best[idx];
+        return {static_cast<int>(c.algo), c.mapping, c.fused};
+    }
+    return default_candidate(plan->k, v);
+}
+
+}  // namespace sepconv
+
+using namespace sepconv;
+
+// ==== C ABI ===========================================================================================
+extern "C" {
+
+const char *sepconv_version(void) { return "sepconv-b200 0.1 (sm_100a)"; }
+
+const char *sepconv_status_str(sepconv_status_t s) {
+    switch (s) {
+        case SEPCONV_OK: return "ok";
+        case SEPCONV_E_INVALID: return "invalid argument";
+        case SEPCONV_E_ALIGN: return "misaligned pointer";
+        case SEPCONV_E_ALIAS: return "input and output overlap";
+        case SEPCONV_E_UNSUPPORTED: return "unsupported";
+        case SEPCONV_E_NOMEM: return "out of memory";
+        case SEPCONV_E_CUDA: return "CUDA error";
+        case SEPCONV_E_NCCL: return "NCCL error";
+    }
+    return "unknown status";
+}
+
+const char *sepconv_last_error(void) { return t_last_error.c_str(); }
+
+uint64_t sepconv_launch_count(void) { return g_launches.load(); }
+
+static sepconv_status_t validate_desc(const sepconv_plan_desc_t *d) {
+    if (!d) return fail(SEPCONV_E_INVALID, "descriptor is NULL");
+    if (d->k > SEPCONV_MAX_K) return fail(SEPCONV_E_UNSUPPORTED, "K=%d exceeds SEPCONV_MAX_K=%d", d->k, SEPCONV_MAX_K);
+    if (d->k < 1) return fail(SEPCONV_E_INVALID, "K=%d must be >= 1", d->k);
+    if (d->n < 1) return fail(SEPCONV_E_INVALID, "n=%lld must be >= 1", (long long)d->n);
+    if (d->h < d->k || d->w < d->k)
+        return fail(SEPCONV_E_INVALID, "image %lldx%lld smaller than kernel width %d (output would be empty)",
+                    (long long)d->h, (long long)d->w, d->k);
+    if (d->h > (1LL << 30) || d->w > (1LL << 30) || d->n > (1LL << 30))
+        return fail(SEPCONV_E_INVALID, "dimension too large");
+    const int64_t ld_in = d->ld_in ? d->ld_in : d->w;
+    const int64_t ld_out = d->ld_out ? d->ld_out : d->w - d->k + 1;
+    if (ld_in < d->w) return fail(SEPCONV_E_INVALID, "ld_in=%lld < w=%lld", (long long)ld_in, (long long)d->w);
+    if (ld_out < d->w - d->k + 1)
+        return fail(SEPCONV_E_INVALID, "ld_out=%lld < w-k+1=%lld", (long long)ld_out, (long long)(d->w - d->k + 1));
+    if (d->ld_in < 0 || d->ld_out < 0) return fail(SEPCONV_E_INVALID, "negative pitch");
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_plan_ex(const sepconv_plan_desc_t *desc, sepconv_plan_t *plan) {
+    clear_error();
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan out-pointer is NULL");
+    *plan = nullptr;
+    sepconv_status_t s = validate_desc(desc);
+    if (s != SEPCONV_OK) return s;
+    DeviceInfo di;
+    s = query_device(desc->device, &di);
+    if (s != SEPCONV_OK) return s;
+    sepconv_plan_s *p = new (std::nothrow) sepconv_plan_s();
+    if (!p) return fail(SEPCONV_E_NOMEM, "host allocation of the plan failed");
+    p->dev = di;
+    p->n = desc->n;
+    p->h = desc->h;
+    p->w = desc->w;
+    p->k = desc->k;
+    p->ld_in = desc->ld_in ? desc->ld_in : desc->w;
+    p->ho = desc->h - desc->k + 1;
+    p->wo = desc->w - desc->k + 1;
+    p->ld_out = desc->ld_out ? desc->ld_out : p->wo;
+    DeviceGuard guard(di.device);
+    cudaError_t e = cudaEventCreateWithFlags(&p->last_work, cudaEventDisableTiming);
+    if (e != cudaSuccess) {
+        delete p;
+        return cuda_fail(e, "cudaEventCreate");
+    }
+    *plan = p;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_plan(int64_t H, int64_t W, int K, sepconv_plan_t *plan) {
+    sepconv_plan_desc_t d;
+    std::memset(&d, 0, sizeof d);
+    d.n = 1;
+    d.h = H;
+    d.w = W;
+    d.k = K;
+    d.device = -1;
+    return sepconv_plan_ex(&d, plan);
+}
+
+void sepconv_destroy(sepconv_plan_t plan) {
+    if (!plan) return;
+    DeviceGuard guard(plan->dev.device);
+    if (plan->last_work) cudaEventSynchronize(plan->last_work);
+    cudaDeviceSynchronize();
+    sepconv_comm_destroy_internal(plan);
+    if (plan->buf) cudaFree(plan->buf);
+    for (int i = 0; i < 2; ++i) {
+        if (plan->hin[i]) cudaFree(plan->hin[i]);
+        if (plan->hout[i]) cudaFree(plan->hout[i]);
+        if (plan->hbuf[i]) cudaFree(plan->hbuf[i]);
+    }
+    for (auto &s : plan->hstream)
+        if (s) cudaStreamDestroy(s);
+    for (auto &row : plan->hev)
+        for (auto &ev : row)
+            if (ev) cudaEventDestroy(ev);
+    if (plan->last_work) cudaEventDestroy(plan->last_work);
+    delete plan;
+}
+
+sepconv_status_t sepconv_out_shape(sepconv_plan_t plan, int64_t *Ho, int64_t *Wo) {
+    clear_error();
+    if (!plan || !Ho || !Wo) return fail(SEPCONV_E_INVALID, "NULL argument");
+    *Ho = plan->ho;
+    *Wo = plan->wo;
+    return SEPCONV_OK;
+}
+
+static sepconv_status_t check_io(sepconv_plan_t plan, const float *in, const float *out) {
+    if (!in || !out) return fail(SEPCONV_E_INVALID, "in/out must be non-NULL device pointers");
+    if (!aligned(in, 4) || !aligned(out, 4)) return fail(SEPCONV_E_ALIGN, "in/out must be 4-byte aligned");
+    const long long ein = extent_floats(plan->n, plan->h * plan->ld_in, plan->h, plan->ld_in, plan->w);
+    const long long eout = extent_floats(plan->n, plan->ho * plan->ld_out, plan->ho, plan->ld_out, plan->wo);
+    const uintptr_t a0 = reinterpret_cast<uintptr_t>(in), a1 = a0 + ein * 4;
+    const uintptr_t b0 = reinterpret_cast<uintptr_t>(out), b1 = b0 + eout * 4;
+    if (a0 < b1 && b0 < a1) return fail(SEPCONV_E_ALIAS, "input and output ranges overlap (in-place is not supported)");
+    return SEPCONV_OK;
+}
+
+static sepconv_status_t check_choice(const sepconv_choice_t *c) {
+    if (!c) return fail(SEPCONV_E_INVALID, "choice is NULL");
+    if (c->algo != SEPCONV_2D && c->algo != SEPCONV_SEPARABLE)
+        return fail(SEPCONV_E_INVALID, "choice.algo must be SEPCONV_2D or SEPCONV_SEPARABLE");
+    if (c->mapping != SEPCONV_MAP_DIRECT && c->mapping != SEPCONV_MAP_TMA)
+        return fail(SEPCONV_E_INVALID, "choice.mapping must be DIRECT or TMA");
+    return SEPCONV_OK;
+}
+
+static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const float *kernel, float *out,
+                                     const Candidate &c, cudaStream_t st) {
+    sepconv_status_t s = check_io(plan, in, out);
+    if (s != SEPCONV_OK) return s;
+    s = check_kernel(kernel, plan->k);
+    if (s != SEPCONV_OK) return s;
+    DeviceGuard guard(plan->dev.device);
+    if (c.algo == SEPCONV_SEPARABLE && !c.fused) {
+        s = ensure_buf(plan);
+        if (s != SEPCONV_OK) return s;
+    }
+    Geometry g = plan_geometry(plan);
+    // the unfused buffer for a whole-image launch is [n][h][ld_buf] (rows = ho + K - 1 = h)
+    s = launch_candidate(plan, g, in, out, kernel, c, plan->buf, plan->ld_buf, st);
+    if (s != SEPCONV_OK) return s;
+    cudaEventRecord(plan->last_work, st);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_run(sepconv_plan_t plan, const float *in, const float *kernel, float *out,
+                             sepconv_variant_t variant, sepconv_stream_t stream) {
+    clear_error();
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
+    if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
+        return fail(SEPCONV_E_INVALID, "variant %d is not 2D / SEPARABLE / AUTO", (int)variant);
+    return run_resolved(plan, in, kernel, out, resolve(plan, variant), static_cast<cudaStream_t>(stream));
+}
+
+sepconv_status_t sepconv_run_choice(sepconv_plan_t plan, const float *in, const float *kernel, float *out,
+                                    const sepconv_choice_t *choice, sepconv_stream_t stream) {
+    clear_error();
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
+    sepconv_status_t s = check_choice(choice);
+    if (s != SEPCONV_OK) return s;
+    Candidate c{static_cast<int>(choice->algo), choice->mapping, choice->algo == SEPCONV_SEPARABLE ? choice->fused : 0};
+    return run_resolved(plan, in, kernel, out, c, static_cast<cudaStream_t>(stream));
+}
+
+sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t variant, sepconv_choice_t *choice) {
+    clear_error();
+    if (!plan || !choice) return fail(SEPCONV_E_INVALID, "NULL argument");
+    if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
+        return fail(SEPCONV_E_INVALID, "bad variant");
+    const int idx = variant == SEPCONV_2D ? 0 : variant == SEPCONV_SEPARABLE ? 1 : 2;
+    if (plan->tuned) {
+        *choice = plan->best[idx];
+    } else {
+        Candidate c = resolve(plan, variant);
+        std::memset(choice, 0, sizeof *choice);
+        choice->algo = static_cast<sepconv_variant_t>(c.algo);
+        choice->mapping = c.mapping;
+        choice->fused = c.fused;
+        choice->warps = kNW;
+        choice->ctas_per_sm = 1;
+    }
+    return SEPCONV_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,222 @@
+// sepconv_band.cpp -- row-band partition of one image across G GPUs (one process per
+// GPU) with the one-sided (K-1)-row input halo exchanged by NCCL send/recv.
+//
+// The paper splits one output matrix into a first and second part across devices
+// and has every task write a sub-region of one big buffer;
+// here that split is G row bands.  Windows extend to +y, so
+// band g needs K-1 input rows owned by band g+1 and nothing from band g-1.
+//
+// NCCL is loaded at run time with dlopen: the libnccl.so.2 already in the process
+// (PyTorch's) when there is one, so the process never holds two NCCLs; else
+// $SEPCONV_NCCL_LIB.  The C ABI therefore does not depend on NCCL at link time.
+#include <cuda_runtime.h>
+#include <dlfcn.h>
+
+#include <cstdlib>
+#include <cstring>
+#include <mutex>
+
+#include "sepconv_internal.h"
+
+using namespace sepconv;
+
+namespace {
+
+// the subset of the NCCL ABI we use (stable since NCCL 2.7)
+typedef int nccl_result_t;
+typedef void *nccl_comm_t;
+struct nccl_unique_id_t {
+    char internal[SEPCONV_NCCL_ID_BYTES];
+};
+constexpr int kNcclFloat32 = 7;
+
+struct NcclApi {
+    bool ok = false;
+    std::string why;
+    nccl_result_t (*GetUniqueId)(nccl_unique_id_t *) = nullptr;
+    nccl_result_t (*CommInitRank)(nccl_comm_t *, int, nccl_unique_id_t, int) = nullptr;
+    nccl_result_t (*CommDestroy)(nccl_comm_t) = nullptr;
+    nccl_result_t (*Send)(const void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
+    nccl_result_t (*Recv)(void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
+    nccl_result_t (*GroupStart)() = nullptr;
+    nccl_result_t (*GroupEnd)() = nullptr;
+    const char *(*GetErrorString)(nccl_result_t) = nullptr;
+};
+
+NcclApi &nccl() {
+    static NcclApi api;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        void *h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD);
+        if (!h) {
+            const char *env = std::getenv("SEPCONV_NCCL_LIB");
+            h = dlopen(env ? env : "libnccl.so.2", RTLD_NOW | RTLD_GLOBAL);
+        }
+        if (!h) {
+            api.why = std::string("cannot load libnccl.so.2: ") + dlerror();
+            return;
+        }
+#define SC_SYM(field, name)                                                   \
+    api.field = reinterpret_cast<decltype(api.field)>(dlsym(h, name));        \
+    if (!api.field) {                                                         \
+        api.why = std::string("libnccl.so.2 lacks ") + name;                  \
+        return;                                                               \
+    }
+        SC_SYM(GetUniqueId, "ncclGetUniqueId");
+        SC_SYM(CommInitRank, "ncclCommInitRank");
+        SC_SYM(CommDestroy, "ncclCommDestroy");
+        SC_SYM(Send, "ncclSend");
+        SC_SYM(Recv, "ncclRecv");
+        SC_SYM(GroupStart, "ncclGroupStart");
+        SC_SYM(GroupEnd, "ncclGroupEnd");
+        SC_SYM(GetErrorString, "ncclGetErrorString");
+#undef SC_SYM
+        api.ok = true;
+    });
+    return api;
+}
+
+sepconv_status_t nccl_fail(nccl_result_t r, const char *what) {
+    NcclApi &a = nccl();
+    return fail(SEPCONV_E_NCCL, "%s: %s", what, a.GetErrorString ? a.GetErrorString(r) : "error");
+}
+
+}  // namespace
+
+void sepconv_comm_destroy_internal(sepconv_plan_t plan) {
+    if (plan->comm && nccl().ok) nccl().CommDestroy(static_cast<nccl_comm_t>(plan->comm));
+    plan->comm = nullptr;
+    if (plan->comm_stream) cudaStreamDestroy(plan->comm_stream);
+    if (plan->ev_in) cudaEventDestroy(plan->ev_in);
+    if (plan->ev_halo) cudaEventDestroy(plan->ev_halo);
+    plan->comm_stream = nullptr;
+    plan->ev_in = plan->ev_halo = nullptr;
+}
+
+extern "C" {
+
+sepconv_status_t sepconv_band(int64_t H, int K, int G, int g, int64_t *out_row0, int64_t *out_rows,
+                              int64_t *in_rows_owned, int64_t *in_rows_alloc) {
+    if (K < 1 || K > SEPCONV_MAX_K) return fail(K > SEPCONV_MAX_K ? SEPCONV_E_UNSUPPORTED : SEPCONV_E_INVALID,
+                                                "K=%d out of range", K);
+    if (H < K) return fail(SEPCONV_E_INVALID, "H=%lld < K=%d", (long long)H, K);
+    if (G < 1 || g < 0 || g >= G) return fail(SEPCONV_E_INVALID, "band %d of %d", g, G);
+    const int64_t ho = H - K + 1;
+    if (G > 1 && ho / G < K - 1)
+        return fail(SEPCONV_E_INVALID, "bands of %lld rows are thinner than the K-1=%d halo",
+                    (long long)(ho / G), K - 1);
+    if (G > ho) return fail(SEPCONV_E_INVALID, "more bands (%d) than output rows (%lld)", G, (long long)ho);
+    const int64_t r0 = ho * g / G, r1 = ho * (g + 1) / G;
+    if (out_row0) *out_row0 = r0;
+    if (out_rows) *out_rows = r1 - r0;
+    if (in_rows_alloc) *in_rows_alloc = r1 - r0 + K - 1;
+    if (in_rows_owned) *in_rows_owned = (g == G - 1) ? (r1 - r0 + K - 1) : (r1 - r0);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_nccl_unique_id(unsigned char id[SEPCONV_NCCL_ID_BYTES]) {
+    if (!id) return fail(SEPCONV_E_INVALID, "id is NULL");
+    NcclApi &a = nccl();
+    if (!a.ok) return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
+    nccl_unique_id_t u;
+    nccl_result_t r = a.GetUniqueId(&u);
+    if (r != 0) return nccl_fail(r, "ncclGetUniqueId");
+    std::memcpy(id, u.internal, SEPCONV_NCCL_ID_BYTES);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[SEPCONV_NCCL_ID_BYTES], int nranks,
+                                   int rank) {
+    if (!plan || !id) return fail(SEPCONV_E_INVALID, "NULL argument");
+    if (nranks < 1 || rank < 0 || rank >= nranks) return fail(SEPCONV_E_INVALID, "rank %d of %d", rank, nranks);
+    if (plan->n != 1) return fail(SEPCONV_E_INVALID, "row bands split a single image (plan has n=%lld)", (long long)plan->n);
+    NcclApi &a = nccl();
+    if (!a.ok) return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
+    int prev = -1;
+    cudaGetDevice(&prev);
+    SC_CUDA(cudaSetDevice(plan->dev.device));
+    sepconv_comm_destroy_internal(plan);
+    SC_CUDA(cudaStreamCreateWithFlags(&plan->comm_stream, cudaStreamNonBlocking));
+    SC_CUDA(cudaEventCreateWithFlags(&plan->ev_in, cudaEventDisableTiming));
+    SC_CUDA(cudaEventCreateWithFlags(&plan->ev_halo, cudaEventDisableTiming));
+    nccl_unique_id_t u;
+    std::memcpy(u.internal, id, SEPCONV_NCCL_ID_BYTES);
+    nccl_comm_t comm = nullptr;
+    nccl_result_t r = a.CommInitRank(&comm, nranks, u, rank);
+    if (prev >= 0) cudaSetDevice(prev);
+    if (r != 0) return nccl_fail(r, "ncclCommInitRank");
+    plan->comm = comm;
+    plan->nranks = nranks;
+    plan->rank = rank;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const float *kernel, float *out_band,
+                                  sepconv_variant_t variant, sepconv_stream_t stream) {
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
+    if (!plan->comm) return fail(SEPCONV_E_INVALID, "sepconv_comm_init has not been called on this plan");
+    if (!in_band || !out_band) return fail(SEPCONV_E_INVALID, "NULL band pointer");
+    if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
+        return fail(SEPCONV_E_INVALID, "bad variant");
+    sepconv_status_t s = check_kernel(kernel, plan->k);
+    if (s != SEPCONV_OK) return s;
+    NcclApi &a = nccl();
+    const int K = plan->k;
+    const bool last = plan->rank == plan->nranks - 1;
+    const int halo = K - 1;
+    const int64_t ho = plan->ho;   // this band's output rows (plan h = in_rows_alloc)
+    if (!last && ho < halo) return fail(SEPCONV_E_INVALID, "band thinner than the halo");
+
+    int prev = -1;
+    cudaGetDevice(&prev);
+    if (prev != plan->dev.device) SC_CUDA(cudaSetDevice(plan->dev.device));
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    const Candidate c = resolve(plan, variant);
+    if (c.algo == SEPCONV_SEPARABLE && !c.fused) {
+        s = ensure_buf(plan);
+        if (s != SEPCONV_OK) return s;
+    }
+
+    // 1. the exchange (comm stream, after the caller's writes to in_band on `st`)
+    SC_CUDA(cudaEventRecord(plan->ev_in, st));
+    SC_CUDA(cudaStreamWaitEvent(plan->comm_stream, plan->ev_in, 0));
+    if (halo > 0 && plan->nranks > 1) {
+        const size_t cnt = static_cast<size_t>(halo) * plan->ld_in;
+        nccl_comm_t comm = static_cast<nccl_comm_t>(plan->comm);
+        nccl_result_t r = a.GroupStart();
+        if (r == 0 && plan->rank > 0)        // my first K-1 rows complete band rank-1
+            r = a.Send(in_band, cnt, kNcclFloat32, plan->rank - 1, comm, plan->comm_stream);
+        if (r == 0 && !last)                 // rank+1's first K-1 rows complete my band
+            r = a.Recv(in_band + ho * plan->ld_in, cnt, kNcclFloat32, plan->rank + 1, comm, plan->comm_stream);
+        nccl_result_t r2 = a.GroupEnd();
+        if (r != 0) return nccl_fail(r, "ncclSend/ncclRecv");
+        if (r2 != 0) return nccl_fail(r2, "ncclGroupEnd");
+    }
+    SC_CUDA(cudaEventRecord(plan->ev_halo, plan->comm_stream));
+
+    // 2. interior rows: need only owned input rows, overlap the exchange
+    Geometry g = plan_geometry(plan);
+    const int64_t interior = last ? ho : ho - halo;
+    if (interior > 0) {
+        Geometry gi = g;
+        gi.row_begin = 0;
+        gi.rows = static_cast<int>(interior);
+        s = launch_candidate(plan, gi, in_band, out_band, kernel, c, plan->buf, plan->ld_buf, st);
+        if (s != SEPCONV_OK) return s;
+    }
+    // 3. tail rows after the halo has landed (and, on every rank, after our send
+    //    has read in_band, so the caller may reuse it in stream order)
+    SC_CUDA(cudaStreamWaitEvent(st, plan->ev_halo, 0));
+    if (!last && halo > 0) {
+        Geometry gt = g;
+        gt.row_begin = static_cast<int>(interior);
+        gt.rows = halo;
+        s = launch_candidate(plan, gt, in_band, out_band, kernel, c, plan->buf, plan->ld_buf, st);
+        if (s != SEPCONV_OK) return s;
+    }
+    SC_CUDA(cudaEventRecord(plan->last_work, st));
+    if (prev >= 0 && prev != plan->dev.device) cudaSetDevice(prev);
+    return SEPCONV_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,108 @@
+// sepconv_internal.h -- plan object and helpers shared by the host-side C++ files.
+#pragma once
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <atomic>
+#include <cstdarg>
+#include <cstdint>
+#include <map>
+#include <string>
+#include <utility>
+
+#include "../../include/sepconv.h"
+#include "sepconv_launch.h"
+
+namespace sepconv {
+
+// ---- errors --------------------------------------------------------------------------
+sepconv_status_t fail(sepconv_status_t st, const char *fmt, ...);
+sepconv_status_t cuda_fail(cudaError_t e, const char *what);
+extern std::atomic<uint64_t> g_launches;
+
+#define SC_CUDA(call)                                              \
+    do {                                                           \
+        cudaError_t _e = (call);                                   \
+        if (_e != cudaSuccess) return ::sepconv::cuda_fail(_e, #call); \
+    } while (0)
+
+// ---- geometry of one launch sequence -----------------------------------------------------
+// A set of nimg images of in_rows x in_cols (pitch ld_in, image stride in_img),
+// producing output rows [row_begin, row_begin + rows) of each image's
+// (in_rows-K+1) x (in_cols-K+1) valid region (pitch ld_out, stride out_img).
+struct Geometry {
+    int K;
+    int nimg;
+    int in_rows, in_cols;
+    long long ld_in, in_img;
+    int out_cols;
+    long long ld_out, out_img;
+    int row_begin, rows;
+};
+
+struct Candidate {
+    int algo;      // SEPCONV_2D / SEPCONV_SEPARABLE
+    int mapping;   // SEPCONV_MAP_DIRECT / SEPCONV_MAP_TMA
+    int fused;     // separable only
+};
+
+struct TensorMapCache {
+    std::map<std::pair<uintptr_t, long long>, CUtensorMap> maps;   // key: (base, shape hash)
+};
+
+struct DeviceInfo {
+    int device = -1;
+    int sms = 0;
+    int major = 0, minor = 0;
+    size_t l2 = 0;
+    size_t smem_optin = 0;
+    std::string name;
+};
+
+}  // namespace sepconv
+
+struct sepconv_plan_s {
+    sepconv::DeviceInfo dev;
+    int64_t n = 1, h = 0, w = 0;
+    int k = 0;
+    int64_t ld_in = 0, ld_out = 0, ho = 0, wo = 0;
+
+    // unfused-separable workspace: the paper's `buffer` [H][W-K+1]
+    float *buf = nullptr;
+    int64_t ld_buf = 0;
+    size_t buf_floats = 0;
+
+    // tuned choices: [0] 2D, [1] SEPARABLE, [2] AUTO
+    bool tuned = false;
+    sepconv_choice_t best[3] = {};
+
+    sepconv::TensorMapCache tmaps;
+    cudaEvent_t last_work = nullptr;
+
+    // NCCL (row bands)
+    void *comm = nullptr;
+    int nranks = 1, rank = 0;
+    cudaStream_t comm_stream = nullptr;
+    cudaEvent_t ev_in = nullptr, ev_halo = nullptr;
+
+    // host-resident pipeline
+    cudaStream_t hstream[3] = {nullptr, nullptr, nullptr};
+    cudaEvent_t hev[4][2] = {};
+    float *hin[2] = {nullptr, nullptr};
+    float *hout[2] = {nullptr, nullptr};
+    float *hbuf[2] = {nullptr, nullptr};
+    int64_t hchunk_rows = 0;
+};
+
+namespace sepconv {
+// core launcher shared by run / run_host / run_band / tune
+sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const float *in, float *out,
+                                  const float *kernel, const Candidate &c, float *buf, long long ld_buf,
+                                  cudaStream_t st);
+Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v);
+sepconv_status_t check_kernel(const float *kernel, int K);
+Geometry plan_geometry(sepconv_plan_t plan);
+sepconv_status_t ensure_buf(sepconv_plan_t plan);
+}  // namespace sepconv
+
+void sepconv_comm_destroy_internal(sepconv_plan_t plan);   // sepconv_band.cpp

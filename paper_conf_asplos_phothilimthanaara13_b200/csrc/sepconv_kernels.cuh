@@ -1,0 +1,428 @@
+// sepconv_kernels.cuh -- sm_100a kernels for SeparableConvolution (Fig. 1,
+// P:354-408).  Included only by the per-op kernel translation units.
+//
+// Kernel family:
+//   stream_kernel<K, OP, MAP>  column-strip streaming kernels.  Each warp owns a
+//       strip of 32*V output columns (V = 4 per thread) and walks down the rows
+//       of its CTA's row range.  OP selects what a warp does with each input row:
+//         OP_ROWS  ConvolveRows: buf[r][c] = sum_i k_i In[r][c+i]
+//         OP_COLS  ConvolveColumns over buf rows held in a K-slot
+//                  register ring: out[q][c] = sum_j k_j buf[q+j][c]
+//         OP_SEP   both, fused: the row pass result goes straight into the ring
+//                  (the paper's `buffer`, never touches HBM)
+//       MAP_TMA stages SR-row x (32V + K-1)-column boxes of In (halo included)
+//       into a per-warp shared-memory ring by cp.async.bulk.tensor + mbarrier;
+//       MAP_DIRECT(_VEC) reads each thread's window straight from global memory
+//       through L1 (4- or 16-byte loads).
+//   conv2d_kernel<K, MAP>  Convolve2D: each output row is the sum over
+//       j of K-tap dot products of input row q+j with weight row w_j = fl(k_j k_i).
+//
+// Arithmetic order (R6, fixed for every mapping, tile and GPU count):
+//   ROWS/SEP:  b = k_0*x_0; b = fma(k_i, x_i, b) for i = 1..K-1
+//   COLS/SEP:  a = k_0*b_q; a = fma(k_j, b_{q+j}, a) for j = 1..K-1
+//   2D:        p_j = w_j0*x_0; p_j = fma(w_ji, x_i, p_j); a = p_0; a = a + p_j
+// so fused and unfused separable are bitwise identical.
+#pragma once
+#include <cuda.h>
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "sepconv_params.h"
+
+namespace sepconv {
+
+// ---- PTX helpers ----------------------------------------------------------------
+__device__ __forceinline__ uint32_t smem_u32(const void *p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+__device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
+
+__device__ __forceinline__ void fence_barrier_init() {
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t *bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+                 : "memory");
+}
+
+__device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity) {
+    const uint32_t addr = smem_u32(bar);
+    uint32_t done;
+    do {
+        asm volatile(
+            "{\n\t.reg .pred p;\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\t"
+            "selp.u32 %0, 1, 0, p;\n\t}"
+            : "=r"(done)
+            : "r"(addr), "r"(parity)
+            : "memory");
+    } while (!done);
+}
+
+// Orders this warp's earlier generic-proxy shared-memory reads before a following
+// TMA (async-proxy) write into the same stage.
+__device__ __forceinline__ void fence_proxy_async_smem() {
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+
+__device__ __forceinline__ void tma_load_3d(void *dst, const CUtensorMap *map, uint64_t *bar, int c0, int c1,
+                                            int c2) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
+        "[%0], [%1, {%3, %4, %5}], [%2];" ::"r"(smem_u32(dst)),
+        "l"(reinterpret_cast<uint64_t>(map)), "r"(smem_u32(bar)), "r"(c0), "r"(c1), "r"(c2)
+        : "memory");
+}
+
+__device__ __forceinline__ void prefetch_tmap(const CUtensorMap *map) {
+    asm volatile("prefetch.tensormap [%0];" ::"l"(reinterpret_cast<uint64_t>(map)) : "memory");
+}
+
+__device__ __forceinline__ float4 ld_shared4(const float *p) {
+    return *reinterpret_cast<const float4 *>(p);
+}
+
+// Store V=4 consecutive floats of one output row when `ok` (uniform per step).
+// Branch-free: every case is a predicated st.global, because a branch inside
+// the unrolled step body makes ptxas move the weights from uniform registers
+// into vector registers, and FFMA R,R,R,R issues ~30% slower than FFMA R,R,UR,R
+// on B200 (profiles/r01_ubench_ffma.txt).  16-byte stores when the row address
+// is 16-byte aligned (c is a multiple of 4, so the alignment is warp-uniform),
+// 2 x 8-byte when it is 8-byte aligned, 4 x 4-byte otherwise and at the ragged
+// right edge (per-element guards).
+__device__ __forceinline__ void store_out4(float *rowp, int c, int out_cols, const float (&v)[V], bool ok) {
+    float *ptr = rowp + c;
+    const unsigned a = static_cast<unsigned>(reinterpret_cast<uintptr_t>(ptr)) & 15u;
+    const bool full = c + V <= out_cols;
+    const unsigned p16 = ok && full && a == 0;
+    const unsigned p8 = ok && full && a == 8;
+    const unsigned ps = ok && !(full && (a & 7) == 0);
+    const unsigned e0 = ps && c < out_cols;
+    const unsigned e1 = ps && c + 1 < out_cols, e2 = ps && c + 2 < out_cols, e3 = ps && c + 3 < out_cols;
+    asm volatile(
+        "{\n\t.reg .pred q16, q8, q0, q1, q2, q3;\n\t"
+        "setp.ne.u32 q16, %5, 0;\n\t"
+        "setp.ne.u32 q8, %6, 0;\n\t"
+        "setp.ne.u32 q0, %7, 0;\n\t"
+        "setp.ne.u32 q1, %8, 0;\n\t"
+        "setp.ne.u32 q2, %9, 0;\n\t"
+        "setp.ne.u32 q3, %10, 0;\n\t"
+        "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+        "@q8 st.global.v2.f32 [%0], {%1, %2};\n\t"
+        "@q8 st.global.v2.f32 [%0+8], {%3, %4};\n\t"
+        "@q0 st.global.f32 [%0], %1;\n\t"
+        "@q1 st.global.f32 [%0+4], %2;\n\t"
+        "@q2 st.global.f32 [%0+8], %3;\n\t"
+        "@q3 st.global.f32 [%0+12], %4;\n\t}"
+        ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(p16), "r"(p8), "r"(e0), "r"(e1), "r"(e2),
+        "r"(e3)
+        : "memory");
+}
+
+// Direct mapping: this thread's window of XW floats of one input row, read
+// through L1 (neighbouring lanes overlap, so most of it hits).  Branch-free (see
+// store_out4): the row and the columns are clamped into the image instead of
+// guarded.  A clamped row or column only ever feeds an output cell that is not
+// stored (a valid output column c' < in_cols-K+1 reads columns <= in_cols-1; a
+// step past the segment's last input row completes no stored row), so the
+// duplicated values are harmless and every load stays inside the allocation.
+template <int XW, bool VEC>
+__device__ __forceinline__ void load_window_global(float (&x)[(XW + 3) & ~3], const float *__restrict__ img,
+                                                   int r, int c, int in_rows, int in_cols, long long ld_in) {
+    constexpr int XV = (XW + 3) / 4;
+    const float *__restrict__ rowp = img + static_cast<long long>(min(r, in_rows - 1)) * ld_in;
+    if constexpr (VEC) {
+        const int cmax = (in_cols - 1) & ~3;
+#pragma unroll
+        for (int v = 0; v < XV; ++v) {
+            const float4 t = __ldg(reinterpret_cast<const float4 *>(rowp + min(c + 4 * v, cmax)));
+            x[4 * v + 0] = t.x; x[4 * v + 1] = t.y; x[4 * v + 2] = t.z; x[4 * v + 3] = t.w;
+        }
+    } else {
+#pragma unroll
+        for (int e = 0; e < XV * 4; ++e) x[e] = __ldg(rowp + min(c + e, in_cols - 1));
+    }
+}
+
+// ---- the streaming kernel -----------------------------------------------------------
+// One CTA = NW independent warps over NW adjacent 128-column strips; the CTA's
+// share of the (image, CTA-strip, row) space is contiguous, split evenly over
+// the grid so the row granularity is 1 and no CTA idles at the end.
+template <int K, int OP, int MAP, int NW>
+__global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constant__ StreamParams p) {
+    constexpr bool TMA = MAP == MAP_TMA;
+    constexpr bool HALO = OP != OP_COLS;
+    constexpr bool ROWCONV = OP != OP_COLS;
+    constexpr bool RING = OP != OP_ROWS;
+    constexpr int XW = HALO ? V + K - 1 : V;
+    constexpr int XV = (XW + 3) / 4;
+    constexpr int BW = box_width(K, HALO);
+    constexpr int SR = RING ? StreamCfg<K>::SR : 16;
+    constexpr int NS = StreamCfg<K>::NS;
+    constexpr int STAGE = (SR * BW + 31) & ~31;                // floats per stage (128-byte TMA alignment)
+    constexpr int RK = RING ? K : 1;                           // ring slots
+    static_assert(BW <= 256, "TMA box width");
+    static_assert(!RING || SR % K == 0, "ring period must divide the stage");
+
+    extern __shared__ __align__(128) float smem[];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    float *wsm = smem + (TMA ? warp * NS * STAGE : 0);
+    uint64_t *wbar = reinterpret_cast<uint64_t *>(smem + NW * NS * STAGE) + warp * NS;
+
+    if constexpr (TMA) {
+        if (lane == 0) {
+            if (warp == 0) prefetch_tmap(&p.tmap);
+#pragma unroll
+            for (int s = 0; s < NS; ++s) mbar_init(&wbar[s], 1);
+            fence_barrier_init();
+        }
+        __syncwarp();
+    }
+
+    const long long u_begin = p.total * blockIdx.x / gridDim.x;
+    const long long u_end = p.total * (blockIdx.x + 1) / gridDim.x;
+    uint32_t kc = 0;                                           // chunks consumed by this warp
+
+    for (long long u = u_begin; u < u_end;) {
+        const long long sidx = u / p.rows;                     // (image, strip) index
+        const int q0 = static_cast<int>(u - sidx * p.rows);
+        const long long seg_end = min(u_end, (sidx + 1) * static_cast<long long>(p.rows));
+        const int nrows = static_cast<int>(seg_end - u);
+        u = seg_end;
+        const int n = static_cast<int>(sidx / p.nstrips);
+        const int s = static_cast<int>(sidx - static_cast<long long>(n) * p.nstrips);
+        const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
+        if (wcol >= p.out_cols) continue;
+        const int c = wcol + lane * V;                         // this thread's first column
+        const int in_row0 = p.row_begin + q0;
+        const int steps = nrows + (RING ? K - 1 : 0);
+        const int nchunks = (steps + SR - 1) / SR;
+        const float *__restrict__ in_img = p.in + n * p.in_img_stride;
+        float *out_rows = p.out + n * p.out_img_stride + static_cast<long long>(in_row0) * p.ld_out;
+
+        if constexpr (TMA) {
+            if (lane == 0) {
+                const int npro = nchunks < NS ? nchunks : NS;
+                for (int ch = 0; ch < npro; ++ch) {
+                    const int st = (kc + ch) % NS;
+                    mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                    tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + ch * SR, n);
+                }
+            }
+        }
+
+        float acc[RK][V];
+#pragma unroll
+        for (int a = 0; a < RK; ++a)
+#pragma unroll
+            for (int e = 0; e < V; ++e) acc[a][e] = 0.f;
+
+        for (int ch = 0; ch < nchunks; ++ch, ++kc) {
+            const int st = kc % NS;
+            const float *stage = wsm + st * STAGE;
+            if constexpr (TMA) mbar_wait(&wbar[st], (kc / NS) & 1);
+#pragma unroll
+            for (int pr = 0; pr < SR; ++pr) {
+                const int t = ch * SR + pr;                    // step = input row - in_row0
+                float x[XV * 4];
+                if constexpr (TMA) {
+#pragma unroll
+                    for (int v = 0; v < XV; ++v) {
+                        const float4 tt = ld_shared4(stage + pr * BW + lane * V + 4 * v);
+                        x[4 * v + 0] = tt.x; x[4 * v + 1] = tt.y; x[4 * v + 2] = tt.z; x[4 * v + 3] = tt.w;
+                    }
+                } else {
+                    load_window_global<XW, MAP == MAP_DIRECT_VEC>(x, in_img, in_row0 + t, c, p.in_rows,
+                                                                 p.in_cols, p.ld_in);
+                }
+                float b[V];
+                if constexpr (ROWCONV) {
+#pragma unroll
+                    for (int e = 0; e < V; ++e) {
+                        b[e] = p.k[0] * x[e];
+#pragma unroll
+                        for (int i = 1; i < K; ++i) b[e] = fmaf(p.k[i], x[e + i], b[e]);
+                    }
+                } else {
+#pragma unroll
+                    for (int e = 0; e < V; ++e) b[e] = x[e];
+                }
+                if constexpr (RING) {
+                    constexpr int dummy = 0; (void)dummy;
+#pragma unroll
+                    for (int j = 0; j < K; ++j) {
+                        const int slot = ((pr - j) % K + K) % K;
+#pragma unroll
+                        for (int e = 0; e < V; ++e)
+                            acc[slot][e] = (j == 0) ? p.k[0] * b[e] : fmaf(p.k[j], b[e], acc[slot][e]);
+                    }
+                    const int q = t - (K - 1);                 // output row completed by this step
+                    store_out4(out_rows + static_cast<long long>(q) * p.ld_out, c, p.out_cols, acc[(pr + 1) % K],
+                               static_cast<unsigned>(q) < static_cast<unsigned>(nrows));
+                } else {
+                    store_out4(out_rows + static_cast<long long>(t) * p.ld_out, c, p.out_cols, b, t < nrows);
+                }
+            }
+            if constexpr (TMA) {
+                __syncwarp();
+                if (lane == 0 && ch + NS < nchunks) {
+                    fence_proxy_async_smem();
+                    mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                    tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + (ch + NS) * SR, n);
+                }
+            }
+        }
+    }
+}
+
+template <int K, int OP, int MAP, int NW>
+constexpr size_t stream_smem_bytes() {
+    constexpr bool TMA = MAP == MAP_TMA;
+    constexpr bool HALO = OP != OP_COLS;
+    constexpr bool RING = OP != OP_ROWS;
+    constexpr int SR = RING ? StreamCfg<K>::SR : 16;
+    constexpr int NS = StreamCfg<K>::NS;
+    return TMA ? static_cast<size_t>(NW) * NS * ((SR * box_width(K, HALO) + 31) & ~31) * 4 + NW * NS * 8 : 0;
+}
+
+// ---- Convolve2D ------------------------------------------------------------------------
+// Per output row q: a = sum_j (sum_i w_ji x_{q+j, c+i}).  TMA mapping keeps a
+// per-warp ring of NS stages of SR rows; rows [q, q+K-1] must be resident, a
+// stage is refilled once q has passed it.
+template <int K, int MAP, int NW>
+__global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constant__ Conv2DParams p) {
+    constexpr bool TMA = MAP == MAP_TMA;
+    constexpr int XW = V + K - 1;
+    constexpr int XV = (XW + 3) / 4;
+    constexpr int BW = box_width(K, true);
+    constexpr int SR = Conv2DCfg<K>::SR;
+    constexpr int NS = Conv2DCfg<K>::NS;
+    constexpr int STAGE = SR * BW;
+    static_assert((STAGE * 4) % 128 == 0, "TMA destinations must be 128-byte aligned");
+    constexpr int RING_ROWS = NS * SR;
+
+    extern __shared__ __align__(128) float smem[];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    float *wsm = smem + (TMA ? warp * NS * STAGE : 0);
+    uint64_t *wbar = reinterpret_cast<uint64_t *>(smem + NW * NS * STAGE) + warp * NS;
+    if constexpr (TMA) {
+        if (lane == 0) {
+            if (warp == 0) prefetch_tmap(&p.tmap);
+#pragma unroll
+            for (int s = 0; s < NS; ++s) mbar_init(&wbar[s], 1);
+            fence_barrier_init();
+        }
+        __syncwarp();
+    }
+
+    const long long u_begin = p.total * blockIdx.x / gridDim.x;
+    const long long u_end = p.total * (blockIdx.x + 1) / gridDim.x;
+    uint32_t kc = 0;
+
+    for (long long u = u_begin; u < u_end;) {
+        const long long sidx = u / p.rows;
+        const int q0 = static_cast<int>(u - sidx * p.rows);
+        const long long seg_end = min(u_end, (sidx + 1) * static_cast<long long>(p.rows));
+        const int nrows = static_cast<int>(seg_end - u);
+        u = seg_end;
+        const int n = static_cast<int>(sidx / p.nstrips);
+        const int s = static_cast<int>(sidx - static_cast<long long>(n) * p.nstrips);
+        const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;
+        if (wcol >= p.out_cols) continue;
+        const int c = wcol + lane * V;
+        const int in_row0 = p.row_begin + q0;
+        const int nchunks = (nrows + K - 1 + SR - 1) / SR;
+        const float *__restrict__ in_img = p.in + n * p.in_img_stride;
+        float *out_rows = p.out + n * p.out_img_stride + static_cast<long long>(in_row0) * p.ld_out;
+        const uint32_t kc0 = kc;
+        int waited = 0;
+
+        if constexpr (TMA) {
+            if (lane == 0) {
+                const int npro = nchunks < NS ? nchunks : NS;
+                for (int ch = 0; ch < npro; ++ch) {
+                    const int st = (kc0 + ch) % NS;
+                    mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                    tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + ch * SR, n);
+                }
+            }
+        }
+        const int ring_base = static_cast<int>(kc0 % NS) * SR;     // ring row of segment row 0
+
+        for (int q = 0; q < nrows; ++q) {
+            if constexpr (TMA) {
+                const int need = (q + K - 1) / SR;
+                while (waited <= need) {
+                    const uint32_t g = kc0 + waited;
+                    mbar_wait(&wbar[g % NS], (g / NS) & 1);
+                    ++waited;
+                }
+            }
+            float a[V];
+            int rr = ring_base + q;
+            if (rr >= RING_ROWS) rr -= RING_ROWS * (rr / RING_ROWS);
+#pragma unroll
+            for (int j = 0; j < K; ++j) {
+                float x[XV * 4];
+                if constexpr (TMA) {
+                    const float *rowp = wsm + rr * BW + lane * V;
+#pragma unroll
+                    for (int v = 0; v < XV; ++v) {
+                        const float4 tt = ld_shared4(rowp + 4 * v);
+                        x[4 * v + 0] = tt.x; x[4 * v + 1] = tt.y; x[4 * v + 2] = tt.z; x[4 * v + 3] = tt.w;
+                    }
+                    rr = (rr + 1 == RING_ROWS) ? 0 : rr + 1;
+                } else {
+                    load_window_global<XW, MAP == MAP_DIRECT_VEC>(x, in_img, in_row0 + q + j, c, p.in_rows,
+                                                                 p.in_cols, p.ld_in);
+                }
+#pragma unroll
+                for (int e = 0; e < V; ++e) {
+                    float pj = p.w[j * K] * x[e];
+#pragma unroll
+                    for (int i = 1; i < K; ++i) pj = fmaf(p.w[j * K + i], x[e + i], pj);
+                    a[e] = (j == 0) ? pj : a[e] + pj;
+                }
+            }
+            store_out4(out_rows + static_cast<long long>(q) * p.ld_out, c, p.out_cols, a, true);
+            if constexpr (TMA) {
+                // rows < q+1 are dead; a stage is free once q+1 crosses its end
+                if ((q + 1) % SR == 0) {
+                    const int done_chunk = (q + 1) / SR - 1;
+                    const int next = done_chunk + NS;
+                    __syncwarp();
+                    if (lane == 0 && next < nchunks) {
+                        const int st = (kc0 + done_chunk) % NS;
+                        fence_proxy_async_smem();
+                        mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                        tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + next * SR, n);
+                    }
+                }
+            }
+        }
+        if constexpr (TMA) {
+            // consume (wait on) any chunk issued but not needed by the last row
+            const int issued = nchunks;
+            while (waited < issued) {
+                const uint32_t g = kc0 + waited;
+                mbar_wait(&wbar[g % NS], (g / NS) & 1);
+                ++waited;
+            }
+        }
+        kc = kc0 + nchunks;
+    }
+}
+
+template <int K, int MAP, int NW>
+constexpr size_t conv2d_smem_bytes() {
+    return MAP == MAP_TMA ? static_cast<size_t>(NW) * Conv2DCfg<K>::NS * Conv2DCfg<K>::SR * box_width(K, true) * 4 +
+                     NW * Conv2DCfg<K>::NS * 8
+               : 0;
+}
+
+}  // namespace sepconv

@@ -1,0 +1,32 @@
+// sepconv_util.cu -- utility kernels: synthetic fill for the tuner and an L2 flush
+// (a write of a buffer larger than L2, used between timed runs).
+#include "sepconv_kernels.cuh"
+#include "sepconv_launch.h"
+
+namespace sepconv {
+namespace {
+__global__ void fill_pattern_kernel(float *dst, long long n, unsigned seed) {
+    for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n; i += (long long)gridDim.x * blockDim.x) {
+        unsigned long long z = (unsigned long long)i + ((unsigned long long)seed << 32) + 0x9E3779B97F4A7C15ull;
+        z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+        z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+        z ^= z >> 31;
+        dst[i] = (float)(z >> 40) * (1.0f / 16777216.0f);
+    }
+}
+__global__ void l2_flush_kernel(float4 *dst, long long n4) {
+    const float4 v = make_float4(0.f, 0.f, 0.f, 0.f);
+    for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n4; i += (long long)gridDim.x * blockDim.x)
+        dst[i] = v;
+}
+}  // namespace
+
+cudaError_t launch_fill_pattern(float *dst, long long n, unsigned seed, cudaStream_t st) {
+    fill_pattern_kernel<<<148 * 8, 256, 0, st>>>(dst, n, seed);
+    return cudaGetLastError();
+}
+cudaError_t launch_l2_flush(float *scratch, long long n, cudaStream_t st) {
+    l2_flush_kernel<<<148 * 8, 256, 0, st>>>(reinterpret_cast<float4 *>(scratch), n / 4);
+    return cudaGetLastError();
+}
+}  // namespace sepconv

@@ -1,0 +1,311 @@
+"""Thin Python binding of libsepconv.so (include/sepconv.h) -- argument marshalling only.
+
+Every step of SeparableConvolution runs in the library's sm_100a kernels; this
+module converts Python/torch arguments to the C ABI's plain pointers and sizes
+and turns status codes into exceptions.  There is no fallback: if the library
+is missing or cannot be loaded, :func:`lib` raises.
+
+The names follow the C ABI (``sepconv_plan`` -> :func:`plan`, ``sepconv_run`` ->
+:meth:`Plan.run`, ``sepconv_tune`` -> :meth:`Plan.tune`, ...).
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import threading
+from dataclasses import dataclass
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libsepconv.so")
+
+SEPCONV_2D, SEPCONV_SEPARABLE, SEPCONV_AUTO = 0, 1, 2
+MAP_DIRECT, MAP_TMA = 0, 1
+TUNE_FORCE, TUNE_NO_L2_FLUSH = 1, 2
+MAX_K = 17
+NCCL_ID_BYTES = 128
+VARIANTS = {"2d": SEPCONV_2D, "separable": SEPCONV_SEPARABLE, "auto": SEPCONV_AUTO}
+
+STATUS = {0: "OK", -1: "E_INVALID", -2: "E_ALIGN", -3: "E_ALIAS", -4: "E_UNSUPPORTED",
+          -5: "E_NOMEM", -6: "E_CUDA", -7: "E_NCCL"}
+
+
+class SepconvError(RuntimeError):
+    def __init__(self, status: int, where: str, detail: str):
+        self.status = status
+        self.code = STATUS.get(status, str(status))
+        super().__init__(f"{where}: {self.code}: {detail}")
+
+
+class _Desc(ctypes.Structure):
+    _fields_ = [("n", ctypes.c_int64), ("h", ctypes.c_int64), ("w", ctypes.c_int64), ("k", ctypes.c_int),
+                ("ld_in", ctypes.c_int64), ("ld_out", ctypes.c_int64), ("device", ctypes.c_int)]
+
+
+class _Choice(ctypes.Structure):
+    _fields_ = [("algo", ctypes.c_int), ("mapping", ctypes.c_int), ("fused", ctypes.c_int),
+                ("warps", ctypes.c_int), ("ctas_per_sm", ctypes.c_int), ("median_us", ctypes.c_float)]
+
+
+class _TuneOpts(ctypes.Structure):
+    _fields_ = [("reps", ctypes.c_int), ("cache_path", ctypes.c_char_p), ("flags", ctypes.c_int)]
+
+
+@dataclass(frozen=True)
+class Choice:
+    algo: int
+    mapping: int
+    fused: int
+    warps: int = 8
+    ctas_per_sm: int = 1
+    median_us: float = 0.0
+
+    @property
+    def name(self) -> str:
+        a = "2d" if self.algo == SEPCONV_2D else ("sep-fused" if self.fused else "sep-unfused")
+        return a + ("-tma" if self.mapping == MAP_TMA else "-direct")
+
+    def _c(self) -> _Choice:
+        return _Choice(self.algo, self.mapping, self.fused, self.warps, self.ctas_per_sm, self.median_us)
+
+    @staticmethod
+    def _from(c: _Choice) -> "Choice":
+        return Choice(c.algo, c.mapping, c.fused, c.warps, c.ctas_per_sm, float(c.median_us))
+
+
+_lib = None
+_lock = threading.Lock()
+
+
+def lib() -> ctypes.CDLL:
+    """Load libsepconv.so (RuntimeError if it is absent: there is no CPU fallback)."""
+    global _lib
+    with _lock:
+        if _lib is not None:
+            return _lib
+        if not os.path.exists(LIB_PATH):
+            raise RuntimeError(f"{LIB_PATH} is missing: build it with "
+                               "`python -m paper_conf_asplos_phothilimthanaara13_b200.build`")
+        L = ctypes.CDLL(LIB_PATH)
+        P, I, I64, F = ctypes.c_void_p, ctypes.c_int, ctypes.c_int64, ctypes.c_float
+        pI64 = ctypes.POINTER(ctypes.c_int64)
+        sig = {
+            "sepconv_plan": (I, [I64, I64, I, ctypes.POINTER(P)]),
+            "sepconv_plan_ex": (I, [ctypes.POINTER(_Desc), ctypes.POINTER(P)]),
+            "sepconv_destroy": (None, [P]),
+            "sepconv_out_shape": (I, [P, pI64, pI64]),
+            "sepconv_run": (I, [P, P, P, P, I, P]),
+            "sepconv_run_choice": (I, [P, P, P, P, ctypes.POINTER(_Choice), P]),
+            "sepconv_run_host": (I, [P, P, P, P, I, P]),
+            "sepconv_tune": (I, [P, ctypes.POINTER(_TuneOpts), ctypes.POINTER(_Choice)]),
+            "sepconv_get_choice": (I, [P, I, ctypes.POINTER(_Choice)]),
+            "sepconv_num_candidates": (I, [P]),
+            "sepconv_get_candidate": (I, [P, I, ctypes.POINTER(_Choice)]),
+            "sepconv_band": (I, [I64, I, I, I, pI64, pI64, pI64, pI64]),
+            "sepconv_nccl_unique_id": (I, [ctypes.c_char_p]),
+            "sepconv_comm_init": (I, [P, ctypes.c_char_p, I, I]),
+            "sepconv_run_band": (I, [P, P, P, P, I, P]),
+            "sepconv_status_str": (ctypes.c_char_p, [I]),
+            "sepconv_last_error": (ctypes.c_char_p, []),
+            "sepconv_version": (ctypes.c_char_p, []),
+            "sepconv_launch_count": (ctypes.c_uint64, []),
+        }
+        for name, (res, args) in sig.items():
+            fn = getattr(L, name)
+            fn.restype = res
+            fn.argtypes = args
+        _ = F
+        _lib = L
+        return L
+
+
+def _check(st: int, where: str):
+    if st != 0:
+        raise SepconvError(st, where, (lib().sepconv_last_error() or b"").decode())
+
+
+def version() -> str:
+    return lib().sepconv_version().decode()
+
+
+def launch_count() -> int:
+    """Kernels this library has launched in this process."""
+    return int(lib().sepconv_launch_count())
+
+
+def exported_symbols():
+    return ["sepconv_plan", "sepconv_plan_ex", "sepconv_destroy", "sepconv_out_shape", "sepconv_run",
+            "sepconv_run_choice", "sepconv_run_host", "sepconv_tune", "sepconv_get_choice",
+            "sepconv_num_candidates", "sepconv_get_candidate", "sepconv_band", "sepconv_nccl_unique_id",
+            "sepconv_comm_init", "sepconv_run_band", "sepconv_status_str", "sepconv_last_error",
+            "sepconv_version", "sepconv_launch_count"]
+
+
+def _variant(v) -> int:
+    if isinstance(v, str):
+        return VARIANTS[v.lower()]
+    return int(v)
+
+
+def _kernel_buf(kernel, K: int):
+    k = np.ascontiguousarray(np.asarray(kernel, dtype=np.float32).reshape(-1))
+    if k.size != K:
+        raise ValueError(f"kernel has {k.size} taps, plan expects K={K}")
+    return k
+
+
+def _ptr(x) -> int:
+    """Raw pointer from an int, a torch tensor (device or host) or a numpy array."""
+    if x is None:
+        return 0
+    if isinstance(x, int):
+        return x
+    if hasattr(x, "data_ptr"):
+        return int(x.data_ptr())
+    if isinstance(x, np.ndarray):
+        return int(x.ctypes.data)
+    raise TypeError(f"cannot take a pointer of {type(x)!r}")
+
+
+def _stream(stream) -> int:
+    if stream is None:
+        import torch
+        return int(torch.cuda.current_stream().cuda_stream)
+    if isinstance(stream, int):
+        return stream
+    return int(stream.cuda_stream)
+
+
+def band(H: int, K: int, G: int, g: int):
+    """sepconv_band: (out_row0, out_rows, in_rows_owned, in_rows_alloc) of band g of G."""
+    vals = [ctypes.c_int64() for _ in range(4)]
+    _check(lib().sepconv_band(H, K, G, g, *[ctypes.byref(v) for v in vals]), "sepconv_band")
+    return tuple(int(v.value) for v in vals)
+
+
+def nccl_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(NCCL_ID_BYTES)
+    _check(lib().sepconv_nccl_unique_id(buf), "sepconv_nccl_unique_id")
+    return buf.raw
+
+
+class Plan:
+    """Owns a sepconv_plan_t.  Shapes: in [n][h][ld_in], out [n][h-k+1][ld_out], float32."""
+
+    def __init__(self, h: int, w: int, k: int, n: int = 1, ld_in: int = 0, ld_out: int = 0, device: int = -1):
+        self.n, self.h, self.w, self.k = int(n), int(h), int(w), int(k)
+        self.ld_in = int(ld_in) or self.w
+        self.ld_out = int(ld_out) or (self.w - self.k + 1)
+        self._h = ctypes.c_void_p()
+        d = _Desc(self.n, self.h, self.w, self.k, int(ld_in), int(ld_out), int(device))
+        _check(lib().sepconv_plan_ex(ctypes.byref(d), ctypes.byref(self._h)), "sepconv_plan_ex")
+
+    # -- lifecycle --
+    def close(self):
+        if self._h and self._h.value:
+            lib().sepconv_destroy(self._h)
+            self._h = ctypes.c_void_p()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *exc):
+        self.close()
+
+    @property
+    def handle(self):
+        return self._h
+
+    def out_shape(self):
+        ho, wo = ctypes.c_int64(), ctypes.c_int64()
+        _check(lib().sepconv_out_shape(self._h, ctypes.byref(ho), ctypes.byref(wo)), "sepconv_out_shape")
+        return int(ho.value), int(wo.value)
+
+    # -- running --
+    def run(self, inp, kernel, out, variant="auto", stream=None):
+        """sepconv_run on device buffers (torch CUDA tensors or raw pointers), async on `stream`."""
+        k = _kernel_buf(kernel, self.k)
+        _check(lib().sepconv_run(self._h, _ptr(inp), k.ctypes.data, _ptr(out), _variant(variant),
+                                 _stream(stream)), "sepconv_run")
+        return out
+
+    def run_choice(self, inp, kernel, out, choice: Choice, stream=None):
+        k = _kernel_buf(kernel, self.k)
+        c = choice._c()
+        _check(lib().sepconv_run_choice(self._h, _ptr(inp), k.ctypes.data, _ptr(out), ctypes.byref(c),
+                                        _stream(stream)), "sepconv_run_choice")
+        return out
+
+    def run_host(self, inp, kernel, out, variant="auto", stream=None):
+        """sepconv_run_host on HOST buffers (numpy arrays or pinned torch CPU tensors); synchronous."""
+        k = _kernel_buf(kernel, self.k)
+        _check(lib().sepconv_run_host(self._h, _ptr(inp), k.ctypes.data, _ptr(out), _variant(variant),
+                                      _stream(stream)), "sepconv_run_host")
+        return out
+
+    # -- tuning --
+    def tune(self, reps: int = 20, cache_path: str | None = None, force: bool = False,
+             no_l2_flush: bool = False) -> Choice:
+        flags = (TUNE_FORCE if force else 0) | (TUNE_NO_L2_FLUSH if no_l2_flush else 0)
+        opts = _TuneOpts(int(reps), cache_path.encode() if cache_path else None, flags)
+        out = _Choice()
+        _check(lib().sepconv_tune(self._h, ctypes.byref(opts), ctypes.byref(out)), "sepconv_tune")
+        return Choice._from(out)
+
+    def get_choice(self, variant="auto") -> Choice:
+        out = _Choice()
+        _check(lib().sepconv_get_choice(self._h, _variant(variant), ctypes.byref(out)), "sepconv_get_choice")
+        return Choice._from(out)
+
+    def candidates(self):
+        res = []
+        for i in range(lib().sepconv_num_candidates(self._h)):
+            c = _Choice()
+            _check(lib().sepconv_get_candidate(self._h, i, ctypes.byref(c)), "sepconv_get_candidate")
+            res.append(Choice._from(c))
+        return res
+
+    # -- row bands --
+    def comm_init(self, unique_id: bytes, nranks: int, rank: int):
+        if len(unique_id) != NCCL_ID_BYTES:
+            raise ValueError("NCCL unique id must be 128 bytes")
+        _check(lib().sepconv_comm_init(self._h, unique_id, int(nranks), int(rank)), "sepconv_comm_init")
+
+    def run_band(self, in_band, kernel, out_band, variant="auto", stream=None):
+        k = _kernel_buf(kernel, self.k)
+        _check(lib().sepconv_run_band(self._h, _ptr(in_band), k.ctypes.data, _ptr(out_band), _variant(variant),
+                                      _stream(stream)), "sepconv_run_band")
+        return out_band
+
+
+def plan(H: int, W: int, K: int) -> Plan:
+    """sepconv_plan: one dense H x W image, width-K kernel, current device."""
+    return Plan(H, W, K)
+
+
+def plan_ex(n: int, h: int, w: int, k: int, ld_in: int = 0, ld_out: int = 0, device: int = -1) -> Plan:
+    return Plan(h, w, k, n=n, ld_in=ld_in, ld_out=ld_out, device=device)
+
+
+def convolve(inp, kernel, variant="auto", out=None, plan_obj: Plan | None = None, stream=None):
+    """Convenience: torch CUDA float32 [h][w] or [n][h][w] in -> new (or given) out tensor."""
+    import torch
+    if not (inp.is_cuda and inp.dtype == torch.float32):
+        raise TypeError("convolve expects a CUDA float32 tensor")
+    x = inp if inp.dim() == 3 else inp.unsqueeze(0)
+    n, h, w = x.shape
+    if x.stride(-1) != 1 or x.stride(0) != h * x.stride(1):
+        raise ValueError("rows must be contiguous and images packed back to back")
+    K = int(np.asarray(kernel).size)
+    p = plan_obj or Plan(h, w, K, n=n, ld_in=x.stride(1), device=x.device.index)
+    if out is None:
+        out = torch.empty((n, h - K + 1, w - K + 1), dtype=torch.float32, device=x.device)
+    p.run(x, kernel, out, variant, stream)
+    return out if inp.dim() == 3 else out[0]

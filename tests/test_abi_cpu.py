@@ -1,0 +1,96 @@
+"""The C-ABI library without a GPU: it loads, exports every symbol include/sepconv.h
+declares, validates arguments, and its pure-host band arithmetic matches the
+oracle's independent partition (R18).  No compute calls."""
+import os
+import re
+
+import pytest
+
+import oracle
+from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _declared():
+    hdr = open(os.path.join(ROOT, "include", "sepconv.h")).read()
+    return sorted(set(re.findall(r"\b(sepconv_[a-z_]+)\s*\(", hdr)))
+
+
+def test_library_exports_every_declared_symbol():
+    L = sc.lib()
+    declared = _declared()
+    assert len(declared) >= 19
+    for name in declared:
+        assert hasattr(L, name), name
+    assert sorted(sc.exported_symbols()) == declared
+
+
+def test_status_strings_and_version():
+    L = sc.lib()
+    for code in range(-7, 1):
+        assert L.sepconv_status_str(code)
+    assert "sm_100a" in sc.version()
+    assert sc.launch_count() == 0
+
+
+@pytest.mark.parametrize("args,code", [
+    ((16, 16, 0), "E_INVALID"),
+    ((16, 16, 18), "E_UNSUPPORTED"),
+    ((2, 16, 3), "E_INVALID"),
+    ((16, 2, 3), "E_INVALID"),
+])
+def test_plan_validation_before_device(args, code):
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.plan(*args)
+    assert ei.value.code == code
+
+
+def test_plan_ex_pitch_validation():
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.plan_ex(1, 16, 16, 3, ld_in=8)
+    assert ei.value.code == "E_INVALID"
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.plan_ex(1, 16, 16, 3, ld_out=5)
+    assert ei.value.code == "E_INVALID"
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.plan_ex(0, 16, 16, 3)
+    assert ei.value.code == "E_INVALID"
+
+
+def test_plan_without_device_is_unsupported():
+    torch = pytest.importorskip("torch")
+    if torch.cuda.is_available():
+        pytest.skip("has a GPU")
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.plan(64, 64, 3)
+    assert ei.value.code == "E_UNSUPPORTED"
+
+
+@pytest.mark.parametrize("H,K,G", [(64, 3, 1), (64, 3, 2), (100, 5, 3), (16384, 17, 8), (16384, 3, 4), (1001, 9, 7)])
+def test_band_matches_oracle_partition(H, K, G):
+    ho = H - K + 1
+    total_out, owned_sum = 0, 0
+    for g in range(G):
+        r0, rows, owned, alloc = sc.band(H, K, G, g)
+        o0, o1 = oracle.band_rows(ho, G, g)
+        assert (r0, rows) == (o0, o1 - o0)
+        assert alloc == rows + K - 1
+        assert owned == (rows + K - 1 if g == G - 1 else rows)
+        total_out += rows
+        owned_sum += owned
+    assert total_out == ho
+    assert owned_sum == H          # every input row owned by exactly one rank
+
+
+def test_band_rejects_thin_bands():
+    with pytest.raises(sc.SepconvError):
+        sc.band(40, 17, 8, 0)       # 24 output rows / 8 = 3 < K-1 = 16
+    with pytest.raises(sc.SepconvError):
+        sc.band(40, 3, 2, 2)
+    with pytest.raises(sc.SepconvError):
+        sc.band(40, 18, 1, 0)
+
+
+def test_band_single_gpu_is_whole_image():
+    assert sc.band(100, 7, 1, 0) == (0, 94, 100, 100)

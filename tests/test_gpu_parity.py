@@ -1,0 +1,241 @@
+"""GPU parity: the CUDA path through the C ABI vs the CPU oracle, element by element.
+
+Bar (tests/parity.py): max |g - o| / S <= 1e-5 with S = sum |k_i k_j In| (= plain
+relative error for the non-negative benchmark data); bit-exact for integer-valued
+data, delta kernels and shape/halo handling; canaries around every output buffer
+must be untouched.  Runs only on a B200 (-m gpu)."""
+import numpy as np
+import pytest
+
+import oracle
+from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+from paper_conf_asplos_phothilimthanaara13_b200 import synth
+from tests.parity import TOL, rel_error
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+CANDS = [
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_DIRECT, 1),
+    sc.Choice(sc.SEPCONV_2D, sc.MAP_TMA, 0),
+    sc.Choice(sc.SEPCONV_2D, sc.MAP_DIRECT, 0),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 0),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_DIRECT, 0),
+]
+IDS = [c.name for c in CANDS]
+GUARD = 4096          # floats of NaN canary on each side of every output buffer
+
+
+def run_gpu(img, k, choice=None, variant=None, ld_in=0, ld_out=0, off_in=0, off_out=0, plan=None):
+    """Run one convolution through the C ABI with canary-guarded buffers; return out [n][ho][wo]."""
+    x = np.asarray(img, np.float32)
+    if x.ndim == 2:
+        x = x[None]
+    n, h, w = x.shape
+    K = int(np.asarray(k).size)
+    ho, wo = h - K + 1, w - K + 1
+    ld_in = ld_in or w
+    ld_out = ld_out or wo
+    src = np.full((n, h, ld_in), np.nan, np.float32)
+    src[:, :, :w] = x
+    dev_in = torch.empty(off_in + n * h * ld_in + 64, dtype=torch.float32, device="cuda")
+    dev_in[off_in:off_in + src.size] = torch.from_numpy(src.reshape(-1)).cuda()
+    out_len = n * ho * ld_out
+    dev_out = torch.full((2 * GUARD + off_out + out_len,), float("nan"), dtype=torch.float32, device="cuda")
+    p = plan or sc.Plan(h, w, K, n=n, ld_in=ld_in, ld_out=ld_out)
+    pin = dev_in.data_ptr() + 4 * off_in
+    pout = dev_out.data_ptr() + 4 * (GUARD + off_out)
+    if choice is not None:
+        p.run_choice(pin, k, pout, choice)
+    else:
+        p.run(pin, k, pout, variant or "auto")
+    torch.cuda.synchronize()
+    full = dev_out.cpu().numpy()
+    assert np.all(np.isnan(full[:GUARD + off_out])), "canary before the output was overwritten"
+    assert np.all(np.isnan(full[GUARD + off_out + out_len:])), "canary after the output was overwritten"
+    body = full[GUARD + off_out:GUARD + off_out + out_len].reshape(n, ho, ld_out)
+    if ld_out > wo:
+        assert np.all(np.isnan(body[:, :, wo:])), "pitch padding of the output was written"
+    out = body[:, :, :wo]
+    assert not np.any(np.isnan(out)), "an output cell was not written"
+    return out
+
+
+def check(img, k, out):
+    o, s = oracle.convolve2d(img, k, with_absum=True)
+    err = rel_error(out, o, s)
+    assert err <= TOL, f"max relative error {err:.3e} > {TOL}"
+    return err
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+@pytest.mark.parametrize("shape", [(67, 131), (300, 1100)])
+def test_random_all_widths(choice, shape):
+    h, w = shape
+    img = synth.uniform_image(h, w, seed=100 + h) - np.float32(0.5)
+    for K in range(1, 18):
+        k = synth.random_kernel(K, seed=K, signed=True)
+        out = run_gpu(img, k, choice)[0]
+        check(img, k, out)
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+def test_integer_exact_bitwise(choice):
+    img = synth.integer_image(150, 1030, seed=7)
+    for K in (1, 2, 3, 8, 16, 17):
+        k = synth.integer_kernel(K, seed=K)
+        out = run_gpu(img, k, choice)[0]
+        want = oracle.convolve2d(img, k).astype(np.float32)
+        assert np.array_equal(out, want), f"K={K}"
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+def test_delta_kernel_bitwise(choice):
+    img = synth.uniform_image(90, 260, seed=3)
+    for K in (5, 17):
+        for m in (0, K // 2, K - 1):
+            out = run_gpu(img, synth.delta_kernel(K, m), choice)[0]
+            assert np.array_equal(out, img[m:m + 90 - K + 1, m:m + 260 - K + 1])
+
+
+def test_fused_equals_unfused_and_mappings_agree_bitwise():
+    img = synth.uniform_image(333, 2100, seed=11)
+    for K in (3, 8, 17):
+        k = synth.random_kernel(K, seed=K, signed=True)
+        outs = [run_gpu(img, k, c)[0] for c in CANDS]
+        sep = [o for o, c in zip(outs, CANDS) if c.algo == sc.SEPCONV_SEPARABLE]
+        two = [o for o, c in zip(outs, CANDS) if c.algo == sc.SEPCONV_2D]
+        for o in sep[1:]:
+            assert np.array_equal(o, sep[0])
+        for o in two[1:]:
+            assert np.array_equal(o, two[0])
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+def test_pitched_and_misaligned(choice):
+    img = synth.uniform_image(120, 517, seed=5)
+    for K, ld_in, ld_out, off_in, off_out in ((3, 520, 515, 0, 0), (7, 517, 511, 1, 1), (16, 523, 505, 3, 2),
+                                               (17, 528, 512, 0, 3)):
+        k = synth.random_kernel(K, seed=K)
+        out = run_gpu(img, k, choice, ld_in=ld_in, ld_out=ld_out, off_in=off_in, off_out=off_out)[0]
+        check(img, k, out)
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+def test_batch_equals_single_images(choice):
+    imgs = np.stack([synth.uniform_image(70, 300, seed=50, n=i) for i in range(3)])
+    K = 9
+    k = synth.binomial_kernel(K)
+    batch = run_gpu(imgs, k, choice)
+    for i in range(3):
+        assert np.array_equal(batch[i], run_gpu(imgs[i], k, choice)[0])
+        check(imgs[i], k, batch[i])
+
+
+@pytest.mark.parametrize("choice", CANDS, ids=IDS)
+def test_degenerate_shapes(choice):
+    for h, w, K in ((17, 17, 17), (1, 1, 1), (5, 300, 5), (300, 5, 5), (64, 64, 3), (2, 9000, 2)):
+        img = synth.uniform_image(h, w, seed=h * w)
+        k = synth.random_kernel(K, seed=1)
+        out = run_gpu(img, k, choice)[0]
+        assert out.shape == (h - K + 1, w - K + 1)
+        check(img, k, out)
+
+
+def test_variants_and_auto_default():
+    img = synth.uniform_image(64, 64, seed=0x5EC0000)       # BASELINE config C1
+    k = synth.binomial_kernel(3)
+    for v in ("2d", "separable", "auto"):
+        check(img, k, run_gpu(img, k, variant=v)[0])
+
+
+def test_tune_choice_is_valid_and_cached(tmp_path):
+    cache = str(tmp_path / "tune.jsonl")
+    img = synth.uniform_image(512, 768, seed=9)
+    k = synth.binomial_kernel(11)
+    p = sc.Plan(512, 768, 11)
+    best = p.tune(reps=3, cache_path=cache, force=True)
+    assert best.median_us > 0
+    names = {c.name for c in p.candidates()}
+    assert best.name in names
+    for v in ("2d", "separable", "auto"):
+        c = p.get_choice(v)
+        assert c.median_us > 0
+        assert c.name in names
+    assert p.get_choice("auto").median_us <= min(p.get_choice("2d").median_us, p.get_choice("separable").median_us) * 1.0001
+    check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
+    q = sc.Plan(512, 768, 11)
+    again = q.tune(reps=3, cache_path=cache)                 # cache hit: no re-measurement
+    assert again == best
+
+
+def test_run_host_pipeline():
+    h, w, K = 2500, 16384, 5                                 # 3 row bands of 1024 rows
+    img = synth.uniform_image(h, w, seed=21)
+    k = synth.binomial_kernel(K)
+    src = torch.from_numpy(img).pin_memory()
+    dst = torch.empty((h - K + 1, w - K + 1), dtype=torch.float32).pin_memory()
+    p = sc.Plan(h, w, K)
+    for v in ("separable", "2d"):
+        dst.fill_(float("nan"))
+        p.run_host(src, k, dst, v)
+        check(img, k, dst.numpy())
+
+
+def test_errors():
+    p = sc.Plan(64, 64, 3)
+    buf = torch.zeros(64 * 64 * 2, device="cuda")
+    k = synth.binomial_kernel(3)
+    with pytest.raises(sc.SepconvError) as ei:
+        p.run(buf.data_ptr(), k, buf.data_ptr() + 4 * 100, "auto")
+    assert ei.value.code == "E_ALIAS"
+    with pytest.raises(sc.SepconvError) as ei:
+        p.run(buf.data_ptr() + 2, k, buf.data_ptr() + 4 * 5000, "auto")
+    assert ei.value.code == "E_ALIGN"
+    with pytest.raises(sc.SepconvError) as ei:
+        sc.lib()
+        st = sc.lib().sepconv_run(p.handle, buf.data_ptr(), None, buf.data_ptr() + 4 * 5000, 2, 0)
+        sc._check(st, "sepconv_run")
+    assert ei.value.code == "E_INVALID"
+    with pytest.raises(sc.SepconvError) as ei:
+        p.run(buf.data_ptr(), k, buf.data_ptr() + 4 * 5000, 7)
+    assert ei.value.code == "E_INVALID"
+
+
+def test_launch_count_increases():
+    before = sc.launch_count()
+    img = synth.uniform_image(64, 300, seed=1)
+    run_gpu(img, synth.binomial_kernel(5), CANDS[4])          # unfused: 2 launches
+    assert sc.launch_count() == before + 2
+
+
+# ---- full BASELINE size, the configuration bench.py times, sampled rows --------------------
+@pytest.mark.parametrize("K", [3, 5, 7, 9, 11, 13, 15, 17])
+def test_full_size_16384_sampled_rows(K, _big_image):
+    img, dev_in = _big_image
+    H = W = 16384
+    ho, wo = H - K + 1, W - K + 1
+    k = synth.binomial_kernel(K)
+    p = sc.Plan(H, W, K)
+    out = torch.empty((ho, wo), dtype=torch.float32, device="cuda")
+    rows = sorted({0, 1, 1023, 1024, 8191, ho // 2, ho - 2, ho - 1})
+    for v in ("auto", "2d"):
+        out.fill_(float("nan"))
+        p.run(dev_in, k, out, v)
+        torch.cuda.synchronize()
+        assert not torch.isnan(out).any().item()
+        got = out[rows].cpu().numpy()
+        for i, r in enumerate(rows):
+            o, s = oracle.convolve2d(np.ascontiguousarray(img[r:r + K]), k, with_absum=True)
+            assert rel_error(got[i:i + 1], o, s) <= TOL, (v, r)
+        # property at full size: non-negative data and kernel summing to 1 keep every output in [0, 1)
+        assert float(out.min()) >= 0.0 and float(out.max()) < 1.0
+
+
+@pytest.fixture(scope="module")
+def _big_image():
+    img = synth.uniform_image(16384, 16384, seed=synth.BENCH_SEED_BASE + 3)
+    dev = torch.from_numpy(img).cuda()
+    yield img, dev
+    del dev
