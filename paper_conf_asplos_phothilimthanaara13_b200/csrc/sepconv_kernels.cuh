@@ -52,8 +52,10 @@ __device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t *bar, uint32_t by
 
 __device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity) {
     const uint32_t addr = smem_u32(bar);
-    uint32_t done;
+    uint32_t done, spins = 0;
     do {
+        // a lost transaction would otherwise hang the GPU: fail loudly instead
+        if (++spins == (1u << 26)) __trap();
         asm volatile(
             "{\n\t.reg .pred p;\n\t"
             "mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\t"
@@ -164,6 +166,7 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
     constexpr int BW = box_width(K, HALO);
     constexpr int SR = RING ? StreamCfg<K>::SR : 16;
     constexpr int NS = StreamCfg<K>::NS;
+    constexpr int BOX_BYTES = SR * BW * 4;                     // bytes one TMA box delivers
     constexpr int STAGE = (SR * BW + 31) & ~31;                // floats per stage (128-byte TMA alignment)
     constexpr int RK = RING ? K : 1;                           // ring slots
     static_assert(BW <= 256, "TMA box width");
@@ -210,7 +213,7 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
                 const int npro = nchunks < NS ? nchunks : NS;
                 for (int ch = 0; ch < npro; ++ch) {
                     const int st = (kc + ch) % NS;
-                    mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                    mbar_arrive_expect_tx(&wbar[st], BOX_BYTES);
                     tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + ch * SR, n);
                 }
             }
@@ -272,7 +275,7 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
                 __syncwarp();
                 if (lane == 0 && ch + NS < nchunks) {
                     fence_proxy_async_smem();
-                    mbar_arrive_expect_tx(&wbar[st], STAGE * 4);
+                    mbar_arrive_expect_tx(&wbar[st], BOX_BYTES);
                     tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + (ch + NS) * SR, n);
                 }
             }
