@@ -7,7 +7,7 @@ namespace {
 template <int K, int MAP>
 KernelInfo info_one() {
     return {reinterpret_cast<const void *>(&conv2d_kernel<K, MAP, kNW>), conv2d_smem_bytes<K, MAP, kNW>(),
-            kNW * 32};
+            kNW * 32, Conv2DCfg<K>::SR, 0};
 }
 template <int K, int MAP>
 cudaError_t launch_one(const Conv2DParams &p, int grid, cudaStream_t st) {

@@ -117,7 +117,7 @@ static long long extent_floats(long long nimg, long long img, long long rows, lo
 }
 
 // ---- launching ------------------------------------------------------------------------------------
-static int map_index(bool tma, bool vec16) { return tma ? MAP_TMA : (vec16 ? MAP_DIRECT_VEC : MAP_DIRECT); }
+static int map_index(bool tma, bool vec16) { return tma ? MAP_TMA : (vec16 ? MAP_DIRECT_VEC : MAP_DIRECT); }  // conv2d
 
 static sepconv_status_t prepare_func(const KernelInfo &ki, int dev, const DeviceInfo &di, int *blocks_per_sm) {
     // attribute setting is cheap but not free: cache per (function, device)
@@ -171,9 +171,30 @@ static bool tma_ok(const float *base, long long ld, long long img) {
     return aligned(base, 16) && (ld % 4) == 0 && (img % 4) == 0;
 }
 
-static int grid_for(const DeviceInfo &di, int occ, long long total) {
-    long long g = static_cast<long long>(di.sms) * occ;
-    if (g > total) g = total;
+// Work schedule (SegmentIter in sepconv_kernels.cuh).  Preferred: `parts` row partitions
+// per (image, strip), with the strip index fastest across CTAs, so the CTAs in flight walk
+// a few row windows of the image together (2 MB pages and L2 sets stay hot; neighbouring
+// strips read their shared halo columns at the same time) -- measured +8% at K=3..13 on
+// 16384^2 over the contiguous split.  It leaves at most nimg*nstrips-1 CTA slots idle, so
+// when the (image, strip) count is large relative to the grid the exactly balanced
+// contiguous split (parts = 0) is used instead.  Segments shorter than 4(K-1) rows would
+// spend most of their time on warm-up rows, so the grid shrinks for small images.
+static int schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K, int *parts) {
+    const long long slots = static_cast<long long>(di.sms) * occ;
+    const long long strips = static_cast<long long>(nimg) * nstrips;
+    const long long min_rows = std::max(8, 4 * (K - 1));
+    long long want = std::max<long long>(1, static_cast<long long>(rows) / min_rows);   // parts per strip
+    if (strips <= slots) {
+        long long pp = std::min<long long>(slots / strips, want);
+        const long long used = strips * pp;
+        if (used * 10 >= slots * 9 || pp == want) {             // <= 10% of the slots idle
+            *parts = static_cast<int>(std::max<long long>(pp, 1));
+            return static_cast<int>(std::max<long long>(used, 1));
+        }
+    }
+    *parts = 0;
+    const long long total = strips * rows;
+    long long g = std::min<long long>(slots, std::max<long long>(1, total / min_rows));
     return static_cast<int>(std::max<long long>(g, 1));
 }
 
@@ -181,16 +202,19 @@ static int grid_for(const DeviceInfo &di, int occ, long long total) {
 static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geometry &g, const float *in,
                                          long long ld_in, long long in_img, int in_cols, float *out,
                                          long long ld_out, long long out_img, int out_cols, int rows_total,
-                                         const float *kernel, bool want_tma, cudaStream_t st) {
+                                         const float *kernel, bool want_tma, int cfg, cudaStream_t st) {
     const int K = g.K;
     const bool tma = want_tma && tma_ok(in, ld_in, in_img);
     const bool vec = aligned(in, 16) && (ld_in % 4) == 0 && (in_img % 4) == 0;
-    const int map = map_index(tma, vec);
+    // variant: 0 direct, 1 direct 16-byte, 2.. TMA configurations (stream_geom)
+    const int ntma = stream_variants(op) - 2;
+    const int map = tma ? 2 + std::min(std::max(cfg, 0), ntma - 1) : (vec ? 1 : 0);
     KernelInfo ki = op == OP_ROWS ? stream_rows_info(map, K) : op == OP_COLS ? stream_cols_info(map, K)
                                                                             : stream_sep_info(map, K);
     int occ = 0;
     sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);
     if (s != SEPCONV_OK) return s;
+    if (ki.cps > 0) occ = std::min(occ, ki.cps);
 
     StreamParams p;
     std::memset(&p, 0, sizeof p);
@@ -206,18 +230,20 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     p.row_begin = g.row_begin;
     p.rows = rows_total;
     p.nimg = g.nimg;
-    const int cta_cols = kNW * kWarpCols;
+    const int cta_cols = (ki.threads / 32) * kWarpCols;
     p.nstrips = (out_cols + cta_cols - 1) / cta_cols;
     p.total = static_cast<long long>(g.nimg) * p.nstrips * rows_total;
-    for (int i = 0; i < K; ++i) p.k[i] = kernel[i];
+    p.store8 = aligned(out, 8) && (ld_out % 2) == 0 && (out_img % 2) == 0;
+    for (int i = 0; i < K; ++i) {
+        p.k[i] = kernel[i];
+        p.k2[i] = make_float2(kernel[i], kernel[i]);
+    }
     if (tma) {
-        const bool halo = op != OP_COLS;
-        const int sr = op == OP_ROWS ? 16 : K * std::max(1, 20 / K);
-        s = make_tmap(plan, &p.tmap, in, in_cols, g.in_rows, g.nimg, ld_in, in_img, box_width(K, halo), sr);
+        s = make_tmap(plan, &p.tmap, in, in_cols, g.in_rows, g.nimg, ld_in, in_img, stream_bw(K, op), ki.stage_rows);
         if (s != SEPCONV_OK) return s;
     }
     if (p.total <= 0) return SEPCONV_OK;
-    const int grid = grid_for(plan->dev, occ, p.total);
+    const int grid = schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K, &p.parts);
     cudaError_t e = op == OP_ROWS ? stream_rows_launch(map, K, p, grid, st)
                     : op == OP_COLS ? stream_cols_launch(map, K, p, grid, st)
                                     : stream_sep_launch(map, K, p, grid, st);
@@ -253,6 +279,7 @@ static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const 
     const int cta_cols = kNW * kWarpCols;
     p.nstrips = (g.out_cols + cta_cols - 1) / cta_cols;
     p.total = static_cast<long long>(g.nimg) * p.nstrips * g.rows;
+    p.store8 = aligned(out, 8) && (g.ld_out % 2) == 0 && (g.out_img % 2) == 0;
     // w_ji = fl(k_i * k_j): the outer-product weights of Convolve2D, rounded once
     for (int j = 0; j < K; ++j)
         for (int i = 0; i < K; ++i) p.w[j * K + i] = kernel[i] * kernel[j];
@@ -262,7 +289,7 @@ static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const 
         if (s != SEPCONV_OK) return s;
     }
     if (p.total <= 0) return SEPCONV_OK;
-    const int grid = grid_for(plan->dev, occ, p.total);
+    const int grid = schedule(plan->dev, occ, g.nimg, p.nstrips, g.rows, K, &p.parts);
     cudaError_t e = conv2d_launch(map, K, p, grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "conv2d kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
@@ -288,7 +315,7 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
     if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st);
     if (c.fused)
         return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, st);
+                                g.out_cols, g.rows, kernel, tma, c.config, st);
     // Choice 2 as the paper writes it: ConvolveRows into buffer, then ConvolveColumns.
     // The buffer holds the rows this launch's output rows need: [row_begin, row_begin + rows + K - 1).
     if (!buf) return fail(SEPCONV_E_INVALID, "unfused separable needs a workspace");
@@ -306,7 +333,7 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
         gg.in_rows = g.in_rows - g.row_begin;
         gg.row_begin = 0;
         sepconv_status_t s = launch_stream_op(plan, OP_ROWS, gg, in0, g.ld_in, g.in_img, g.in_cols, buf, ld_buf,
-                                              buf_img, g.out_cols, brows, kernel, tma, st);
+                                              buf_img, g.out_cols, brows, kernel, tma, 0, st);
         if (s != SEPCONV_OK) return s;
     }
     {
@@ -315,22 +342,28 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
         gc.row_begin = 0;
         float *out0 = out + static_cast<long long>(g.row_begin) * g.ld_out;
         return launch_stream_op(plan, OP_COLS, gc, buf, ld_buf, buf_img, g.out_cols, out0, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, st);
+                                g.out_cols, g.rows, kernel, tma, 0, st);
     }
 }
 
 // Static default before tuning (R16): fused separable with TMA for K >= 2
 // (one HBM pass, 2K FMA/px), 2D with TMA for K = 1.
 static Candidate default_candidate(int K, sepconv_variant_t v) {
-    if (v == SEPCONV_2D || (v == SEPCONV_AUTO && K == 1)) return {SEPCONV_2D, SEPCONV_MAP_TMA, 0};
-    return {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1};
+    if (v == SEPCONV_2D || (v == SEPCONV_AUTO && K == 1)) return {SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0};
+    return {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, 0};
+}
+
+int candidate_warps(int K, const Candidate &c) {
+    if (c.algo == SEPCONV_SEPARABLE && c.fused && c.mapping == SEPCONV_MAP_TMA)
+        return stream_sep_info(2 + c.config, K).threads / 32;
+    return kNW;
 }
 
 Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v) {
     const int idx = v == SEPCONV_2D ? 0 : v == SEPCONV_SEPARABLE ? 1 : 2;
     if (plan->tuned) {
         const sepconv_choice_t &c = plan->best[idx];
-        return {static_cast<int>(c.algo), c.mapping, c.fused};
+        return {static_cast<int>(c.algo), c.mapping, c.fused, c.config};
     }
     return default_candidate(plan->k, v);
 }
@@ -468,6 +501,8 @@ static sepconv_status_t check_choice(const sepconv_choice_t *c) {
         return fail(SEPCONV_E_INVALID, "choice.algo must be SEPCONV_2D or SEPCONV_SEPARABLE");
     if (c->mapping != SEPCONV_MAP_DIRECT && c->mapping != SEPCONV_MAP_TMA)
         return fail(SEPCONV_E_INVALID, "choice.mapping must be DIRECT or TMA");
+    if (c->config < 0 || c->config >= kSepTmaConfigs)
+        return fail(SEPCONV_E_INVALID, "choice.config must be in [0, %d)", kSepTmaConfigs);
     return SEPCONV_OK;
 }
 
@@ -505,7 +540,8 @@ sepconv_status_t sepconv_run_choice(sepconv_plan_t plan, const float *in, const 
     if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
     sepconv_status_t s = check_choice(choice);
     if (s != SEPCONV_OK) return s;
-    Candidate c{static_cast<int>(choice->algo), choice->mapping, choice->algo == SEPCONV_SEPARABLE ? choice->fused : 0};
+    Candidate c{static_cast<int>(choice->algo), choice->mapping, choice->algo == SEPCONV_SEPARABLE ? choice->fused : 0,
+                choice->config};
     return run_resolved(plan, in, kernel, out, c, static_cast<cudaStream_t>(stream));
 }
 
@@ -523,7 +559,8 @@ sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t varia
         choice->algo = static_cast<sepconv_variant_t>(c.algo);
         choice->mapping = c.mapping;
         choice->fused = c.fused;
-        choice->warps = kNW;
+        choice->config = c.config;
+        choice->warps = candidate_warps(plan->k, c);
         choice->ctas_per_sm = 1;
     }
     return SEPCONV_OK;

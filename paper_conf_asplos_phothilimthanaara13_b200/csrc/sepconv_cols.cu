@@ -1,24 +1,44 @@
-// sepconv_cols.cu -- instantiations of stream_kernel<K, OP_COLS, MAP, kNW> for K = 1..17 and the
-// three mappings (direct scalar, direct 16-byte, TMA).
+// sepconv_cols.cu -- instantiations of stream_kernel for OP_COLS, K = 1..17, every mapping
+// variant of stream_geom (sepconv_params.h).
 #include "sepconv_kernels.cuh"
 #include "sepconv_launch.h"
 
 namespace sepconv {
 namespace {
-template <int K, int MAP>
+constexpr int NV = stream_variants(OP_COLS);
+template <int K, int V_>
 KernelInfo info_one() {
-    return {reinterpret_cast<const void *>(&stream_kernel<K, OP_COLS, MAP, kNW>),
-            stream_smem_bytes<K, OP_COLS, MAP, kNW>(), kNW * 32};
+    using I = StreamInst<K, OP_COLS, V_>;
+    return {reinterpret_cast<const void *>(I::kernel), I::smem, I::threads, I::G.sr, I::G.cps};
 }
-template <int K, int MAP>
+template <int K, int V_>
 cudaError_t launch_one(const StreamParams &p, int grid, cudaStream_t st) {
-    stream_kernel<K, OP_COLS, MAP, kNW><<<grid, kNW * 32, stream_smem_bytes<K, OP_COLS, MAP, kNW>(), st>>>(p);
+    using I = StreamInst<K, OP_COLS, V_>;
+    I::kernel<<<grid, I::threads, I::smem, st>>>(p);
     return cudaGetLastError();
 }
-using InfoFn = KernelInfo (*)();
-using LaunchFn = cudaError_t (*)(const StreamParams &, int, cudaStream_t);
-#define SEPCONV_ROW(K) {info_one<K, MAP_DIRECT>, info_one<K, MAP_DIRECT_VEC>, info_one<K, MAP_TMA>}
-const InfoFn kInfo[kMaxK][3] = {
+template <int K, int... Vs>
+struct Row {
+    static constexpr KernelInfo (*info[sizeof...(Vs)])() = {info_one<K, Vs>...};
+    static constexpr cudaError_t (*launch[sizeof...(Vs)])(const StreamParams &, int, cudaStream_t) = {launch_one<K, Vs>...};
+};
+template <int K, int... Vs>
+KernelInfo info_dispatch(int v, std::integer_sequence<int, Vs...>) {
+    return Row<K, Vs...>::info[v]();
+}
+template <int K, int... Vs>
+cudaError_t launch_dispatch(int v, const StreamParams &p, int grid, cudaStream_t st, std::integer_sequence<int, Vs...>) {
+    return Row<K, Vs...>::launch[v](p, grid, st);
+}
+using Seq = std::make_integer_sequence<int, NV>;
+using InfoFn = KernelInfo (*)(int);
+using LaunchFn = cudaError_t (*)(int, const StreamParams &, int, cudaStream_t);
+template <int K>
+KernelInfo info_k(int v) { return info_dispatch<K>(v, Seq{}); }
+template <int K>
+cudaError_t launch_k(int v, const StreamParams &p, int grid, cudaStream_t st) { return launch_dispatch<K>(v, p, grid, st, Seq{}); }
+#define SEPCONV_ROW(K) info_k<K>
+const InfoFn kInfo[kMaxK] = {
     SEPCONV_ROW(1),
     SEPCONV_ROW(2),
     SEPCONV_ROW(3),
@@ -37,8 +57,8 @@ const InfoFn kInfo[kMaxK][3] = {
     SEPCONV_ROW(16),
     SEPCONV_ROW(17)};
 #undef SEPCONV_ROW
-#define SEPCONV_ROW(K) {launch_one<K, MAP_DIRECT>, launch_one<K, MAP_DIRECT_VEC>, launch_one<K, MAP_TMA>}
-const LaunchFn kLaunch[kMaxK][3] = {
+#define SEPCONV_ROW(K) launch_k<K>
+const LaunchFn kLaunch[kMaxK] = {
     SEPCONV_ROW(1),
     SEPCONV_ROW(2),
     SEPCONV_ROW(3),
@@ -59,8 +79,8 @@ const LaunchFn kLaunch[kMaxK][3] = {
 #undef SEPCONV_ROW
 }  // namespace
 
-KernelInfo stream_cols_info(int map, int K) { return kInfo[K - 1][map](); }
-cudaError_t stream_cols_launch(int map, int K, const StreamParams &p, int grid, cudaStream_t st) {
-    return kLaunch[K - 1][map](p, grid, st);
+KernelInfo stream_cols_info(int variant, int K) { return kInfo[K - 1](variant); }
+cudaError_t stream_cols_launch(int variant, int K, const StreamParams &p, int grid, cudaStream_t st) {
+    return kLaunch[K - 1](variant, p, grid, st);
 }
 }  // namespace sepconv

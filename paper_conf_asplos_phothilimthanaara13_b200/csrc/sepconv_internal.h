@@ -44,6 +44,7 @@ struct Candidate {
     int algo;      // SEPCONV_2D / SEPCONV_SEPARABLE
     int mapping;   // SEPCONV_MAP_DIRECT / SEPCONV_MAP_TMA
     int fused;     // separable only
+    int config;    // fused + TMA: stage configuration 0..kSepTmaConfigs-1 (stream_geom)
 };
 
 struct TensorMapCache {
@@ -100,6 +101,7 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
                                   const float *kernel, const Candidate &c, float *buf, long long ld_buf,
                                   cudaStream_t st);
 Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v);
+int candidate_warps(int K, const Candidate &c);
 sepconv_status_t check_kernel(const float *kernel, int K);
 Geometry plan_geometry(sepconv_plan_t plan);
 sepconv_status_t ensure_buf(sepconv_plan_t plan);

@@ -27,6 +27,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include <type_traits>
+
 #include "sepconv_params.h"
 
 namespace sepconv {
@@ -85,46 +87,111 @@ __device__ __forceinline__ void prefetch_tmap(const CUtensorMap *map) {
     asm volatile("prefetch.tensormap [%0];" ::"l"(reinterpret_cast<uint64_t>(map)) : "memory");
 }
 
+// Packed FP32 (FFMA2 / FMUL2 on sm_100): two independent IEEE RN operations per
+// instruction -- bitwise the same as two fmaf / two multiplies.
+__device__ __forceinline__ float2 ffma2(float2 a, float2 b, float2 c) {
+    unsigned long long ra = *reinterpret_cast<unsigned long long *>(&a);
+    unsigned long long rb = *reinterpret_cast<unsigned long long *>(&b);
+    unsigned long long rc = *reinterpret_cast<unsigned long long *>(&c), rd;
+    asm("fma.rn.f32x2 %0, %1, %2, %3;" : "=l"(rd) : "l"(ra), "l"(rb), "l"(rc));
+    return *reinterpret_cast<float2 *>(&rd);
+}
+__device__ __forceinline__ float2 fmul2(float2 a, float2 b) {
+    unsigned long long ra = *reinterpret_cast<unsigned long long *>(&a);
+    unsigned long long rb = *reinterpret_cast<unsigned long long *>(&b), rd;
+    asm("mul.rn.f32x2 %0, %1, %2;" : "=l"(rd) : "l"(ra), "l"(rb));
+    return *reinterpret_cast<float2 *>(&rd);
+}
+
 __device__ __forceinline__ float4 ld_shared4(const float *p) {
     return *reinterpret_cast<const float4 *>(p);
 }
 
-// Store V=4 consecutive floats of one output row when `ok` (uniform per step).
-// Branch-free: every case is a predicated st.global, because a branch inside
-// the unrolled step body makes ptxas move the weights from uniform registers
-// into vector registers, and FFMA R,R,R,R issues ~30% slower than FFMA R,R,UR,R
-// on B200 (profiles/r01_ubench_ffma.txt).  16-byte stores when the row address
-// is 16-byte aligned (c is a multiple of 4, so the alignment is warp-uniform),
-// 2 x 8-byte when it is 8-byte aligned, 4 x 4-byte otherwise and at the ragged
-// right edge (per-element guards).
-__device__ __forceinline__ void store_out4(float *rowp, int c, int out_cols, const float (&v)[V], bool ok) {
-    float *ptr = rowp + c;
-    const unsigned a = static_cast<unsigned>(reinterpret_cast<uintptr_t>(ptr)) & 15u;
-    const bool full = c + V <= out_cols;
-    const unsigned p16 = ok && full && a == 0;
-    const unsigned p8 = ok && full && a == 8;
-    const unsigned ps = ok && !(full && (a & 7) == 0);
-    const unsigned e0 = ps && c < out_cols;
-    const unsigned e1 = ps && c + 1 < out_cols, e2 = ps && c + 2 < out_cols, e3 = ps && c + 3 < out_cols;
-    asm volatile(
-        "{\n\t.reg .pred q16, q8, q0, q1, q2, q3;\n\t"
-        "setp.ne.u32 q16, %5, 0;\n\t"
-        "setp.ne.u32 q8, %6, 0;\n\t"
-        "setp.ne.u32 q0, %7, 0;\n\t"
-        "setp.ne.u32 q1, %8, 0;\n\t"
-        "setp.ne.u32 q2, %9, 0;\n\t"
-        "setp.ne.u32 q3, %10, 0;\n\t"
-        "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
-        "@q8 st.global.v2.f32 [%0], {%1, %2};\n\t"
-        "@q8 st.global.v2.f32 [%0+8], {%3, %4};\n\t"
-        "@q0 st.global.f32 [%0], %1;\n\t"
-        "@q1 st.global.f32 [%0+4], %2;\n\t"
-        "@q2 st.global.f32 [%0+8], %3;\n\t"
-        "@q3 st.global.f32 [%0+12], %4;\n\t}"
-        ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(p16), "r"(p8), "r"(e0), "r"(e1), "r"(e2),
-        "r"(e3)
-        : "memory");
-}
+// Output cursor: this thread's 4-column slot of one output row, advanced one row
+// per step.  Stores are branch-free -- every case is a predicated st.global --
+// because a branch inside the unrolled step body makes ptxas move the weights from
+// uniform registers into vector registers, and FFMA R,R,R,R issues ~30% slower than
+// FFMA R,R,UR,R on B200 (profiles/r01_ubench_ffma.txt).  16-byte stores when the
+// row address is 16-byte aligned (c is a multiple of 4, so the alignment is
+// warp-uniform), 2 x 8-byte when it is 8-byte aligned, 4 x 4-byte otherwise and at
+// the ragged right edge (per-element guards computed once per segment).
+struct OutCursor {
+    float *ptr;              // &out[row][c] of the row the next store() writes
+    long long ld;            // row pitch (floats)
+    bool full;               // all 4 columns of this thread are inside the image
+    bool e1, e2, e3, e0;     // column c+e is inside the image
+    __device__ __forceinline__ void init(float *rowp, long long ld_, int c, int out_cols) {
+        ptr = rowp + c;
+        ld = ld_;
+        full = c + V <= out_cols;
+        e0 = c < out_cols;
+        e1 = c + 1 < out_cols;
+        e2 = c + 2 < out_cols;
+        e3 = c + 3 < out_cols;
+    }
+    // Fast path: the warp's 128 columns are inside the image and every row start is
+    // 8-byte aligned (checked by the host).  A 16-byte aligned row is one STG.128 per
+    // lane.  An 8-byte aligned row is re-cut into 16-byte aligned chunks with two
+    // shuffles -- lane l stores (lane l-1's v2, v3, its own v0, v1) -- plus one 8-byte
+    // store at each end of the warp's 512-byte span, so every sector is written once
+    // and whole instead of twice in halves.
+    __device__ __forceinline__ void store_fast(const float (&v)[V], bool ok, int lane) {
+        const unsigned a8 = static_cast<unsigned>(reinterpret_cast<uintptr_t>(ptr)) & 8u;
+        const float u2 = __shfl_up_sync(0xffffffffu, v[2], 1);
+        const float u3 = __shfl_up_sync(0xffffffffu, v[3], 1);
+        const unsigned p16 = ok && a8 == 0;
+        const unsigned pm = ok && a8 != 0 && lane != 0;
+        const unsigned p0 = ok && a8 != 0 && lane == 0;
+        const unsigned p31 = ok && a8 != 0 && lane == 31;
+        asm volatile(
+            "{\n\t.reg .pred q16, qm, q0, q31;\n\t"
+            "setp.ne.u32 q16, %7, 0;\n\t"
+            "setp.ne.u32 qm, %8, 0;\n\t"
+            "setp.ne.u32 q0, %9, 0;\n\t"
+            "setp.ne.u32 q31, %10, 0;\n\t"
+            "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+            "@qm st.global.v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
+            "@q0 st.global.v2.f32 [%0], {%1, %2};\n\t"
+            "@q31 st.global.v2.f32 [%0+8], {%3, %4};\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(u2), "f"(u3), "r"(p16), "r"(pm), "r"(p0),
+            "r"(p31)
+            : "memory");
+        ptr += ld;
+    }
+    template <bool FAST>
+    __device__ __forceinline__ void put(const float (&v)[V], bool ok, int lane) {
+        if constexpr (FAST) store_fast(v, ok, lane);
+        else store(v, ok);
+    }
+    // write v to the cursor row if ok, then move to the next row
+    __device__ __forceinline__ void store(const float (&v)[V], bool ok) {
+        const unsigned a = static_cast<unsigned>(reinterpret_cast<uintptr_t>(ptr)) & 15u;
+        const bool fast = full && (a & 7u) == 0;
+        const unsigned p16 = ok && fast && a == 0;
+        const unsigned p8 = ok && fast && a == 8;
+        const bool ps = ok && !fast;
+        const unsigned q0 = ps && e0, q1 = ps && e1, q2 = ps && e2, q3 = ps && e3;
+        asm volatile(
+            "{\n\t.reg .pred q16, q8, q0, q1, q2, q3;\n\t"
+            "setp.ne.u32 q16, %5, 0;\n\t"
+            "setp.ne.u32 q8, %6, 0;\n\t"
+            "setp.ne.u32 q0, %7, 0;\n\t"
+            "setp.ne.u32 q1, %8, 0;\n\t"
+            "setp.ne.u32 q2, %9, 0;\n\t"
+            "setp.ne.u32 q3, %10, 0;\n\t"
+            "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+            "@q8 st.global.v2.f32 [%0], {%1, %2};\n\t"
+            "@q8 st.global.v2.f32 [%0+8], {%3, %4};\n\t"
+            "@q0 st.global.f32 [%0], %1;\n\t"
+            "@q1 st.global.f32 [%0+4], %2;\n\t"
+            "@q2 st.global.f32 [%0+8], %3;\n\t"
+            "@q3 st.global.f32 [%0+12], %4;\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(p16), "r"(p8), "r"(q0), "r"(q1), "r"(q2),
+            "r"(q3)
+            : "memory");
+        ptr += ld;
+    }
+};
 
 // Direct mapping: this thread's window of XW floats of one input row, read
 // through L1 (neighbouring lanes overlap, so most of it hits).  Branch-free (see
@@ -151,26 +218,71 @@ __device__ __forceinline__ void load_window_global(float (&x)[(XW + 3) & ~3], co
     }
 }
 
+// ---- work decomposition ------------------------------------------------------------------
+// A segment = (image n, CTA strip s, output rows [q0, q0+nrows)); each segment costs K-1
+// warm-up rows.  Two schedules (chosen by the host):
+//   parts > 0: items (n, part j, strip s) with the strip index fastest, CTA b takes items
+//     b, b+grid, ...; part j = rows [j*rows/parts, (j+1)*rows/parts).  Consecutive CTAs walk
+//     the same rows of neighbouring strips, so the CTAs in flight touch a few row windows
+//     (TLB- and L2-friendly: halo columns of neighbouring strips are read at the same time).
+//   parts = 0: CTA b takes the contiguous range [b*total/grid, (b+1)*total/grid) of the
+//     (image, strip, row) space -- exactly balanced, used when items would not divide evenly.
+struct SegmentIter {
+    long long total, u, u_end, item, items;
+    int rows, nstrips, parts;
+    __device__ SegmentIter(long long total_, int rows_, int nstrips_, int parts_, int nimg)
+        : total(total_), rows(rows_), nstrips(nstrips_), parts(parts_) {
+        u = total * blockIdx.x / gridDim.x;
+        u_end = total * (blockIdx.x + 1) / gridDim.x;
+        item = blockIdx.x;
+        items = static_cast<long long>(nimg) * nstrips * (parts > 0 ? parts : 1);
+    }
+    __device__ bool next(int &n, int &s, int &q0, int &nrows) {
+        if (parts > 0) {
+            if (item >= items) return false;
+            s = static_cast<int>(item % nstrips);
+            const long long t = item / nstrips;
+            const int j = static_cast<int>(t % parts);
+            n = static_cast<int>(t / parts);
+            q0 = static_cast<int>(static_cast<long long>(rows) * j / parts);
+            nrows = static_cast<int>(static_cast<long long>(rows) * (j + 1) / parts) - q0;
+            item += gridDim.x;
+            return true;
+        }
+        if (u >= u_end) return false;
+        const long long sidx = u / rows;                       // (image, strip) index
+        q0 = static_cast<int>(u - sidx * rows);
+        const long long seg_end = min(u_end, (sidx + 1) * static_cast<long long>(rows));
+        nrows = static_cast<int>(seg_end - u);
+        u = seg_end;
+        n = static_cast<int>(sidx / nstrips);
+        s = static_cast<int>(sidx - static_cast<long long>(n) * nstrips);
+        return true;
+    }
+};
+
 // ---- the streaming kernel -----------------------------------------------------------
 // One CTA = NW independent warps over NW adjacent 128-column strips; the CTA's
 // share of the (image, CTA-strip, row) space is contiguous, split evenly over
 // the grid so the row granularity is 1 and no CTA idles at the end.
-template <int K, int OP, int MAP, int NW>
-__global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constant__ StreamParams p) {
+template <int K, int OP, int MAP, int NW, int SR_, int NS_, int F2>
+__global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel(const __grid_constant__ StreamParams p) {
     constexpr bool TMA = MAP == MAP_TMA;
     constexpr bool HALO = OP != OP_COLS;
     constexpr bool ROWCONV = OP != OP_COLS;
     constexpr bool RING = OP != OP_ROWS;
     constexpr int XW = HALO ? V + K - 1 : V;
     constexpr int XV = (XW + 3) / 4;
-    constexpr int BW = box_width(K, HALO);
-    constexpr int SR = RING ? StreamCfg<K>::SR : 16;
-    constexpr int NS = StreamCfg<K>::NS;
+    constexpr int BW = stream_bw(K, OP);
+    constexpr int SR = SR_;  // rows per stage
+    constexpr int NS = NS_;
     constexpr int BOX_BYTES = SR * BW * 4;                     // bytes one TMA box delivers
     constexpr int STAGE = (SR * BW + 31) & ~31;                // floats per stage (128-byte TMA alignment)
     constexpr int RK = RING ? K : 1;                           // ring slots
     static_assert(BW <= 256, "TMA box width");
+    static_assert(BW == box_width(K, HALO), "box width");
     static_assert(!RING || SR % K == 0, "ring period must divide the stage");
+    static_assert(!TMA || NW * NS * (STAGE * 4 + 8) <= kSmemPerCta, "shared memory per CTA");
 
     extern __shared__ __align__(128) float smem[];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -187,18 +299,11 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
         __syncwarp();
     }
 
-    const long long u_begin = p.total * blockIdx.x / gridDim.x;
-    const long long u_end = p.total * (blockIdx.x + 1) / gridDim.x;
+    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg);
     uint32_t kc = 0;                                           // chunks consumed by this warp
 
-    for (long long u = u_begin; u < u_end;) {
-        const long long sidx = u / p.rows;                     // (image, strip) index
-        const int q0 = static_cast<int>(u - sidx * p.rows);
-        const long long seg_end = min(u_end, (sidx + 1) * static_cast<long long>(p.rows));
-        const int nrows = static_cast<int>(seg_end - u);
-        u = seg_end;
-        const int n = static_cast<int>(sidx / p.nstrips);
-        const int s = static_cast<int>(sidx - static_cast<long long>(n) * p.nstrips);
+    int n, s, q0, nrows;
+    while (seg.next(n, s, q0, nrows)) {
         const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
         if (wcol >= p.out_cols) continue;
         const int c = wcol + lane * V;                         // this thread's first column
@@ -207,6 +312,9 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
         const int nchunks = (steps + SR - 1) / SR;
         const float *__restrict__ in_img = p.in + n * p.in_img_stride;
         float *out_rows = p.out + n * p.out_img_stride + static_cast<long long>(in_row0) * p.ld_out;
+        // the cursor starts at the row step 0 completes: q = -(K-1) for RING ops
+        OutCursor oc;
+        oc.init(out_rows - (RING ? static_cast<long long>(K - 1) * p.ld_out : 0LL), p.ld_out, c, p.out_cols);
 
         if constexpr (TMA) {
             if (lane == 0) {
@@ -219,6 +327,10 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
             }
         }
 
+        // two copies of the hot loop: the fast store path for warps wholly inside an
+        // image with 8-byte aligned rows, the general one for the ragged edge
+        auto run_chunks = [&](auto fast_tag) {
+        constexpr bool FAST = decltype(fast_tag)::value;
         float acc[RK][V];
 #pragma unroll
         for (int a = 0; a < RK; ++a)
@@ -245,30 +357,60 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
                 }
                 float b[V];
                 if constexpr (ROWCONV) {
+                    if constexpr (F2 >= 2) {
+                        // same per-element order as the scalar path, two columns per instruction:
+                        // xp[m] = (x_2m, x_2m+1) are the loaded pairs, xs[m] = (x_2m+1, x_2m+2) the
+                        // shifted pairs odd taps need (built once per step, shared by both column pairs)
+                        constexpr int NP = (XW + 1) / 2;
+                        float2 xp[NP], xs[NP];
 #pragma unroll
-                    for (int e = 0; e < V; ++e) {
-                        b[e] = p.k[0] * x[e];
+                        for (int m = 0; m < NP; ++m) xp[m] = make_float2(x[2 * m], x[2 * m + 1]);
 #pragma unroll
-                        for (int i = 1; i < K; ++i) b[e] = fmaf(p.k[i], x[e + i], b[e]);
+                        for (int m = 0; m + 1 < NP; ++m) xs[m] = make_float2(x[2 * m + 1], x[2 * m + 2]);
+#pragma unroll
+                        for (int e = 0; e < V; e += 2) {
+                            float2 bb = fmul2(p.k2[0], xp[e / 2]);
+#pragma unroll
+                            for (int i = 1; i < K; ++i)
+                                bb = ffma2(p.k2[i], ((e + i) & 1) ? xs[(e + i) / 2] : xp[(e + i) / 2], bb);
+                            b[e] = bb.x;
+                            b[e + 1] = bb.y;
+                        }
+                    } else {
+#pragma unroll
+                        for (int e = 0; e < V; ++e) {
+                            b[e] = p.k[0] * x[e];
+#pragma unroll
+                            for (int i = 1; i < K; ++i) b[e] = fmaf(p.k[i], x[e + i], b[e]);
+                        }
                     }
                 } else {
 #pragma unroll
                     for (int e = 0; e < V; ++e) b[e] = x[e];
                 }
                 if constexpr (RING) {
-                    constexpr int dummy = 0; (void)dummy;
 #pragma unroll
                     for (int j = 0; j < K; ++j) {
                         const int slot = ((pr - j) % K + K) % K;
+                        if constexpr (F2 >= 1) {
 #pragma unroll
-                        for (int e = 0; e < V; ++e)
-                            acc[slot][e] = (j == 0) ? p.k[0] * b[e] : fmaf(p.k[j], b[e], acc[slot][e]);
+                            for (int e = 0; e < V; e += 2) {
+                                const float2 bb = make_float2(b[e], b[e + 1]);
+                                float2 aa = (j == 0) ? fmul2(p.k2[0], bb)
+                                                     : ffma2(p.k2[j], bb, make_float2(acc[slot][e], acc[slot][e + 1]));
+                                acc[slot][e] = aa.x;
+                                acc[slot][e + 1] = aa.y;
+                            }
+                        } else {
+#pragma unroll
+                            for (int e = 0; e < V; ++e)
+                                acc[slot][e] = (j == 0) ? p.k[0] * b[e] : fmaf(p.k[j], b[e], acc[slot][e]);
+                        }
                     }
                     const int q = t - (K - 1);                 // output row completed by this step
-                    store_out4(out_rows + static_cast<long long>(q) * p.ld_out, c, p.out_cols, acc[(pr + 1) % K],
-                               static_cast<unsigned>(q) < static_cast<unsigned>(nrows));
+                    oc.put<FAST>(acc[(pr + 1) % K], static_cast<unsigned>(q) < static_cast<unsigned>(nrows), lane);
                 } else {
-                    store_out4(out_rows + static_cast<long long>(t) * p.ld_out, c, p.out_cols, b, t < nrows);
+                    oc.put<FAST>(b, t < nrows, lane);
                 }
             }
             if constexpr (TMA) {
@@ -280,18 +422,27 @@ __global__ void __launch_bounds__(NW * 32, 1) stream_kernel(const __grid_constan
                 }
             }
         }
+        };
+        if (p.store8 && wcol + kWarpCols <= p.out_cols) run_chunks(std::true_type{});
+        else run_chunks(std::false_type{});
     }
 }
 
-template <int K, int OP, int MAP, int NW>
+template <int K, int OP, int MAP, int NW, int SR, int NS, int F2>
 constexpr size_t stream_smem_bytes() {
-    constexpr bool TMA = MAP == MAP_TMA;
-    constexpr bool HALO = OP != OP_COLS;
-    constexpr bool RING = OP != OP_ROWS;
-    constexpr int SR = RING ? StreamCfg<K>::SR : 16;
-    constexpr int NS = StreamCfg<K>::NS;
-    return TMA ? static_cast<size_t>(NW) * NS * ((SR * box_width(K, HALO) + 31) & ~31) * 4 + NW * NS * 8 : 0;
+    return MAP == MAP_TMA ? static_cast<size_t>(NW) * NS * ((SR * stream_bw(K, OP) + 31) & ~31) * 4 + NW * NS * 8
+                          : 0;
 }
+
+// The kernel for (K, OP, variant) with the geometry of stream_geom (sepconv_params.h).
+template <int K, int OP, int VARIANT>
+struct StreamInst {
+    static constexpr StreamGeom G = stream_geom(K, OP, VARIANT);
+    static constexpr int MAP = VARIANT >= 2 ? MAP_TMA : VARIANT;
+    static constexpr auto kernel = &stream_kernel<K, OP, MAP, G.nw, G.sr, G.ns, G.f2>;
+    static constexpr size_t smem = stream_smem_bytes<K, OP, MAP, G.nw, G.sr, G.ns, G.f2>();
+    static constexpr int threads = G.nw * 32;
+};
 
 // ---- Convolve2D ------------------------------------------------------------------------
 // Per output row q: a = sum_j (sum_i w_ji x_{q+j, c+i}).  TMA mapping keeps a
@@ -323,18 +474,11 @@ __global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constan
         __syncwarp();
     }
 
-    const long long u_begin = p.total * blockIdx.x / gridDim.x;
-    const long long u_end = p.total * (blockIdx.x + 1) / gridDim.x;
+    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg);
     uint32_t kc = 0;
 
-    for (long long u = u_begin; u < u_end;) {
-        const long long sidx = u / p.rows;
-        const int q0 = static_cast<int>(u - sidx * p.rows);
-        const long long seg_end = min(u_end, (sidx + 1) * static_cast<long long>(p.rows));
-        const int nrows = static_cast<int>(seg_end - u);
-        u = seg_end;
-        const int n = static_cast<int>(sidx / p.nstrips);
-        const int s = static_cast<int>(sidx - static_cast<long long>(n) * p.nstrips);
+    int n, s, q0, nrows;
+    while (seg.next(n, s, q0, nrows)) {
         const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;
         if (wcol >= p.out_cols) continue;
         const int c = wcol + lane * V;
@@ -344,6 +488,8 @@ __global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constan
         float *out_rows = p.out + n * p.out_img_stride + static_cast<long long>(in_row0) * p.ld_out;
         const uint32_t kc0 = kc;
         int waited = 0;
+        OutCursor oc;
+        oc.init(out_rows, p.ld_out, c, p.out_cols);
 
         if constexpr (TMA) {
             if (lane == 0) {
@@ -392,7 +538,7 @@ __global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constan
                     a[e] = (j == 0) ? pj : a[e] + pj;
                 }
             }
-            store_out4(out_rows + static_cast<long long>(q) * p.ld_out, c, p.out_cols, a, true);
+            oc.store(a, true);
             if constexpr (TMA) {
                 // rows < q+1 are dead; a stage is free once q+1 crosses its end
                 if ((q + 1) % SR == 0) {

@@ -1,6 +1,9 @@
 // sepconv_launch.h -- host-side entry points into the kernel translation units.
 #pragma once
 #include <cuda_runtime.h>
+
+#include <utility>
+
 #include "sepconv_params.h"
 
 namespace sepconv {
@@ -11,9 +14,13 @@ struct KernelInfo {
     const void *func;    // the __global__ function (for attributes / occupancy)
     size_t smem;         // dynamic shared memory bytes
     int threads;
+    int stage_rows;      // TMA box height (streaming kernels)
+    int cps;             // CTAs per SM to size the grid for (0 = occupancy limit)
 };
 
-// map: MAP_DIRECT / MAP_DIRECT_VEC / MAP_TMA ; K in [1, 17]
+// streaming kernels: variant = 0 direct, 1 direct 16-byte, 2.. TMA configurations
+// (stream_geom in sepconv_params.h); conv2d: map = MAP_DIRECT / MAP_DIRECT_VEC / MAP_TMA.
+// K in [1, 17]
 KernelInfo stream_rows_info(int map, int K);
 KernelInfo stream_cols_info(int map, int K);
 KernelInfo stream_sep_info(int map, int K);

@@ -2,6 +2,7 @@
 // launcher (plain C++) and the kernels (CUDA).  No device code here.
 #pragma once
 #include <cuda.h>
+#include <cuda_runtime.h>
 #include <stdint.h>
 
 #ifdef __CUDACC__
@@ -36,9 +37,11 @@ struct alignas(64) StreamParams {
     int rows;                    // output rows per image in this launch
     int nimg;
     int nstrips;                 // CTA strips = ceil(out_cols / (warps*128))
-    int pad0;
+    int parts;                   // >0: row partitions per (image, strip), strided schedule; 0: contiguous
+    int store8;                  // 1: out base, ld_out and image stride give 8-byte aligned rows
     long long total;             // nimg * nstrips * rows (work units)
     float k[kMaxK];
+    float2 k2[kMaxK];            // {k_i, k_i}: the same weights as packed-FP32 operands
 };
 
 struct alignas(64) Conv2DParams {
@@ -48,18 +51,58 @@ struct alignas(64) Conv2DParams {
     long long in_img_stride, out_img_stride;
     long long ld_in, ld_out;
     int in_rows, in_cols, out_cols;
-    int row_begin, rows, nimg, nstrips, pad0;
+    int row_begin, rows, nimg, nstrips, parts, store8;
     long long total;
     float w[kMaxK * kMaxK];      // w[j*K + i] = fl(k_i * k_j)
 };
 
 // ---- per-K tile configuration -------------------------------------------------
-template <int K> struct StreamCfg {
-    static constexpr int HALO4 = ((K - 1) + 3) & ~3;            // halo columns, rounded to 16 B
-    static constexpr int M = (20 / K) > 0 ? (20 / K) : 1;
-    static constexpr int SR = K * M;                           // rows per stage: a multiple of K
-    static constexpr int NS = 2;                               // stages per warp
+// Geometry of the streaming kernels (measured on B200 with tools/explore.cu, see
+// profiles/r01_explore_*.txt and DESIGN.md section 6).  Each warp owns a ring of NS
+// stages of SR rows x BW columns in shared memory.  RING ops need SR to be a multiple
+// of K so the register ring's slot indices are compile-time.
+//
+// `variant` selects the mapping: 0 direct (4-byte loads), 1 direct (16-byte loads),
+// 2.. the TMA configurations.  The unfused passes have one TMA configuration; the
+// fused kernel has kSepTmaConfigs, all tuner candidates, because the best one moves
+// with K in ways no simple model predicted (e.g. a 6-row, 2-stage ring reaches 97% of
+// a plain copy at K=3 and K=7 while deeper rings lose 8-12%):
+//   cfg 0  8 warps, SR ~ 6 rows (a multiple of K), 2 stages      (shallow)
+//   cfg 1  8 warps, SR ~ 8 rows, up to 3 stages                   (medium)
+//   cfg 2  K <= 9: 16 warps, SR as cfg 0, up to 4 stages;  K >= 10: 8 warps, SR = K,
+//          as many stages as fit (16 warps would spill the K-slot ring at K >= 10)
+constexpr int kSepTmaConfigs = 3;
+constexpr int kSmemPerCta = 232448 - 1024;     // opt-in limit minus headroom
+
+SEPCONV_HD constexpr int stream_bw(int K, int op) { return 32 * 4 + (op != OP_COLS ? (((K - 1) + 3) & ~3) : 0); }
+SEPCONV_HD constexpr int stage_floats(int sr, int bw) { return (sr * bw + 31) & ~31; }   // 128-byte aligned
+SEPCONV_HD constexpr int ns_fit(int nw, int sr, int bw) { return kSmemPerCta / (nw * (stage_floats(sr, bw) * 4 + 8)); }
+SEPCONV_HD constexpr int clampi(int v, int lo, int hi) { return v < lo ? lo : (v > hi ? hi : v); }
+
+struct StreamGeom {
+    int nw, sr, ns, f2;
+    int cps;       // CTAs per SM the grid is sized for (0 = as many as fit)
 };
+
+SEPCONV_HD constexpr int sep_sr_shallow(int K) { return K >= 6 ? K : K * ((6 + K / 2) / K); }
+SEPCONV_HD constexpr int sep_sr_medium(int K) { return K >= 8 ? K : K * ((8 + K - 1) / K); }
+
+SEPCONV_HD constexpr StreamGeom stream_geom(int K, int op, int variant) {
+    // packed FP32 for the column pass: halves its issue slots (FFMA2 peak is ~8% below FFMA's)
+    return op == OP_SEP
+               ? (variant < 2 ? StreamGeom{8, K >= 8 ? K : K * ((8 + K - 1) / K), 1, K >= 2 ? 1 : 0, 0}
+                  : variant == 2 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1}
+                  : variant == 3 ? StreamGeom{8, sep_sr_medium(K),
+                                              clampi(ns_fit(8, sep_sr_medium(K), stream_bw(K, op)), 1, 3), K >= 2 ? 1 : 0, 1}
+                  : K <= 9 ? StreamGeom{16, sep_sr_shallow(K),
+                                        clampi(ns_fit(16, sep_sr_shallow(K), stream_bw(K, op)), 1, 4), K >= 2 ? 1 : 0, 1}
+                           : StreamGeom{8, K, clampi(ns_fit(8, K, stream_bw(K, op)), 1, 8), 1, 1})
+               : op == OP_ROWS ? StreamGeom{8, 8, clampi(ns_fit(8, 8, stream_bw(K, op)), 1, 8), 0, 0}
+                               : StreamGeom{8, K * ((8 + K - 1) / K),
+                                            clampi(ns_fit(8, K * ((8 + K - 1) / K), stream_bw(K, op)), 1, 8),
+                                            K >= 2 ? 1 : 0, 0};
+}
+SEPCONV_HD constexpr int stream_variants(int op) { return op == OP_SEP ? 2 + kSepTmaConfigs : 3; }
 
 template <int K> struct Conv2DCfg {
     static constexpr int SR = 8;

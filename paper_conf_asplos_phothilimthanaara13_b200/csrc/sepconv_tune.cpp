@@ -27,14 +27,14 @@ namespace {
 
 std::vector<Candidate> candidates(sepconv_plan_t) {
     // fixed order: this is also the tie-break order
-    return {
-        {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1},
-        {SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1},
-        {SEPCONV_2D, SEPCONV_MAP_TMA, 0},
-        {SEPCONV_2D, SEPCONV_MAP_DIRECT, 0},
-        {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 0},
-        {SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 0},
-    };
+    std::vector<Candidate> cs;
+    for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1, 0});
+    cs.push_back({SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0});
+    cs.push_back({SEPCONV_2D, SEPCONV_MAP_DIRECT, 0, 0});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 0, 0});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 0, 0});
+    return cs;
 }
 
 int passes(const Candidate &c) { return (c.algo == SEPCONV_SEPARABLE && !c.fused) ? 2 : 1; }
@@ -48,8 +48,8 @@ std::string cache_key(sepconv_plan_t p) {
 
 std::string choice_json(const sepconv_choice_t &c) {
     char b[160];
-    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%.3f]", (int)c.algo, c.mapping, c.fused, c.warps, c.ctas_per_sm,
-             c.median_us);
+    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%.9g]", (int)c.algo, c.mapping, c.fused, c.config, c.warps,
+             c.ctas_per_sm, c.median_us);
     return b;
 }
 
@@ -57,14 +57,17 @@ bool parse_choice(const std::string &line, const char *field, sepconv_choice_t *
     std::string f = std::string("\"") + field + "\":[";
     size_t pos = line.find(f);
     if (pos == std::string::npos) return false;
-    int algo, map, fused, warps, ctas;
+    int algo, map, fused, config, warps, ctas;
     float us;
-    if (sscanf(line.c_str() + pos + f.size(), "%d,%d,%d,%d,%d,%f", &algo, &map, &fused, &warps, &ctas, &us) != 6)
+    if (sscanf(line.c_str() + pos + f.size(), "%d,%d,%d,%d,%d,%d,%f", &algo, &map, &fused, &config, &warps, &ctas,
+               &us) != 7)
         return false;
+    if (config < 0 || config >= kSepTmaConfigs) return false;
     if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return false;
     c->algo = static_cast<sepconv_variant_t>(algo);
     c->mapping = map;
     c->fused = fused;
+    c->config = config;
     c->warps = warps;
     c->ctas_per_sm = ctas;
     c->median_us = us;
@@ -122,7 +125,8 @@ sepconv_status_t sepconv_get_candidate(sepconv_plan_t plan, int index, sepconv_c
     choice->algo = static_cast<sepconv_variant_t>(cs[index].algo);
     choice->mapping = cs[index].mapping;
     choice->fused = cs[index].fused;
-    choice->warps = kNW;
+    choice->config = cs[index].config;
+    choice->warps = candidate_warps(plan->k, cs[index]);
     choice->ctas_per_sm = 1;
     return SEPCONV_OK;
 }
@@ -237,7 +241,8 @@ sepconv_status_t sepconv_tune(sepconv_plan_t plan, const sepconv_tune_opts_t *op
         o.algo = static_cast<sepconv_variant_t>(c.algo);
         o.mapping = c.mapping;
         o.fused = c.fused;
-        o.warps = kNW;
+        o.config = c.config;
+        o.warps = candidate_warps(plan->k, c);
         o.ctas_per_sm = 1;
         o.median_us = med[bi[s]];
     }

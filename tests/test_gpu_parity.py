@@ -16,7 +16,9 @@ torch = pytest.importorskip("torch")
 pytestmark = pytest.mark.gpu
 
 CANDS = [
-    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 0),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 1),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_DIRECT, 1),
     sc.Choice(sc.SEPCONV_2D, sc.MAP_TMA, 0),
     sc.Choice(sc.SEPCONV_2D, sc.MAP_DIRECT, 0),
@@ -163,7 +165,8 @@ def test_tune_choice_is_valid_and_cached(tmp_path):
         c = p.get_choice(v)
         assert c.median_us > 0
         assert c.name in names
-    assert p.get_choice("auto").median_us <= min(p.get_choice("2d").median_us, p.get_choice("separable").median_us) * 1.0001
+    # ties within 1% go to fewer passes / the lower candidate index (R17)
+    assert p.get_choice("auto").median_us <= min(p.get_choice("2d").median_us, p.get_choice("separable").median_us) * 1.01
     check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
     q = sc.Plan(512, 768, 11)
     again = q.tune(reps=3, cache_path=cache)                 # cache hit: no re-measurement
@@ -206,7 +209,7 @@ def test_errors():
 def test_launch_count_increases():
     before = sc.launch_count()
     img = synth.uniform_image(64, 300, seed=1)
-    run_gpu(img, synth.binomial_kernel(5), CANDS[4])          # unfused: 2 launches
+    run_gpu(img, synth.binomial_kernel(5), CANDS[6])          # unfused: 2 launches
     assert sc.launch_count() == before + 2
 
 
