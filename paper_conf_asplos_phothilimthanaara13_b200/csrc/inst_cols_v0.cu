@@ -1,0 +1,5 @@
+// inst_cols_v0.cu -- stream_kernel instantiations for OP_COLS, variant 0 (see sepconv_inst.cuh).
+#define SEPCONV_OP OP_COLS
+#define SEPCONV_VARIANT 0
+#define SEPCONV_NAME stream_table_cols_v0
+#include "sepconv_inst.cuh"

@@ -209,8 +209,10 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     // variant: 0 direct, 1 direct 16-byte, 2.. TMA configurations (stream_geom)
     const int ntma = stream_variants(op) - 2;
     const int map = tma ? 2 + std::min(std::max(cfg, 0), ntma - 1) : (vec ? 1 : 0);
-    KernelInfo ki = op == OP_ROWS ? stream_rows_info(map, K) : op == OP_COLS ? stream_cols_info(map, K)
-                                                                            : stream_sep_info(map, K);
+    const int store8 = (aligned(out, 16) && (ld_out % 4) == 0 && (out_img % 4) == 0) ? 2
+                       : (aligned(out, 8) && (ld_out % 2) == 0 && (out_img % 2) == 0) ? 1 : 0;
+    const int smode = store8 == 2 ? 2 : 1;
+    KernelInfo ki = stream_info(op, map, K, smode);
     int occ = 0;
     sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);
     if (s != SEPCONV_OK) return s;
@@ -233,7 +235,7 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     const int cta_cols = (ki.threads / 32) * kWarpCols;
     p.nstrips = (out_cols + cta_cols - 1) / cta_cols;
     p.total = static_cast<long long>(g.nimg) * p.nstrips * rows_total;
-    p.store8 = aligned(out, 8) && (ld_out % 2) == 0 && (out_img % 2) == 0;
+    p.store8 = store8;
     for (int i = 0; i < K; ++i) {
         p.k[i] = kernel[i];
         p.k2[i] = make_float2(kernel[i], kernel[i]);
@@ -244,9 +246,7 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     }
     if (p.total <= 0) return SEPCONV_OK;
     const int grid = schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K, &p.parts);
-    cudaError_t e = op == OP_ROWS ? stream_rows_launch(map, K, p, grid, st)
-                    : op == OP_COLS ? stream_cols_launch(map, K, p, grid, st)
-                                    : stream_sep_launch(map, K, p, grid, st);
+    cudaError_t e = stream_launch(op, map, K, smode, p, grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
     return SEPCONV_OK;
@@ -279,7 +279,7 @@ static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const 
     const int cta_cols = kNW * kWarpCols;
     p.nstrips = (g.out_cols + cta_cols - 1) / cta_cols;
     p.total = static_cast<long long>(g.nimg) * p.nstrips * g.rows;
-    p.store8 = aligned(out, 8) && (g.ld_out % 2) == 0 && (g.out_img % 2) == 0;
+    p.store8 = (aligned(out, 8) && (g.ld_out % 2) == 0 && (g.out_img % 2) == 0) ? 1 : 0;   // conv2d: store() only
     // w_ji = fl(k_i * k_j): the outer-product weights of Convolve2D, rounded once
     for (int j = 0; j < K; ++j)
         for (int i = 0; i < K; ++i) p.w[j * K + i] = kernel[i] * kernel[j];
@@ -355,7 +355,7 @@ static Candidate default_candidate(int K, sepconv_variant_t v) {
 
 int candidate_warps(int K, const Candidate &c) {
     if (c.algo == SEPCONV_SEPARABLE && c.fused && c.mapping == SEPCONV_MAP_TMA)
-        return stream_sep_info(2 + c.config, K).threads / 32;
+        return stream_info(OP_SEP, 2 + c.config, K, 1).threads / 32;
     return kNW;
 }
 

@@ -31,6 +31,11 @@
 
 #include "sepconv_params.h"
 
+// cache operator of the output stores ("" = default write-back)
+#ifndef SEPCONV_ST_HINT
+#define SEPCONV_ST_HINT ""
+#endif
+
 namespace sepconv {
 
 // ---- PTX helpers ----------------------------------------------------------------
@@ -149,18 +154,32 @@ struct OutCursor {
             "setp.ne.u32 qm, %8, 0;\n\t"
             "setp.ne.u32 q0, %9, 0;\n\t"
             "setp.ne.u32 q31, %10, 0;\n\t"
-            "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
-            "@qm st.global.v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
-            "@q0 st.global.v2.f32 [%0], {%1, %2};\n\t"
-            "@q31 st.global.v2.f32 [%0+8], {%3, %4};\n\t}"
+            "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+            "@qm st.global" SEPCONV_ST_HINT ".v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
+            "@q0 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
+            "@q31 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
             ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(u2), "f"(u3), "r"(p16), "r"(pm), "r"(p0),
             "r"(p31)
             : "memory");
         ptr += ld;
     }
-    template <bool FAST>
+    // Fastest path: every row start is 16-byte aligned (out base, ld_out and image
+    // stride multiples of 4 floats): one predicated STG.128, nothing else.
+    __device__ __forceinline__ void store_fast16(const float (&v)[V], bool ok) {
+        const unsigned p16 = ok;
+        asm volatile(
+            "{\n\t.reg .pred q16;\n\t"
+            "setp.ne.u32 q16, %5, 0;\n\t"
+            "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(p16)
+            : "memory");
+        ptr += ld;
+    }
+    // MODE 2: 16-byte rows, 1: 8-byte rows, 0: general (ragged edge, 4-byte rows)
+    template <int MODE>
     __device__ __forceinline__ void put(const float (&v)[V], bool ok, int lane) {
-        if constexpr (FAST) store_fast(v, ok, lane);
+        if constexpr (MODE == 2) store_fast16(v, ok);
+        else if constexpr (MODE == 1) store_fast(v, ok, lane);
         else store(v, ok);
     }
     // write v to the cursor row if ok, then move to the next row
@@ -179,7 +198,7 @@ struct OutCursor {
             "setp.ne.u32 q1, %8, 0;\n\t"
             "setp.ne.u32 q2, %9, 0;\n\t"
             "setp.ne.u32 q3, %10, 0;\n\t"
-            "@q16 st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+            "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t"
             "@q8 st.global.v2.f32 [%0], {%1, %2};\n\t"
             "@q8 st.global.v2.f32 [%0+8], {%3, %4};\n\t"
             "@q0 st.global.f32 [%0], %1;\n\t"
@@ -265,7 +284,7 @@ struct SegmentIter {
 // One CTA = NW independent warps over NW adjacent 128-column strips; the CTA's
 // share of the (image, CTA-strip, row) space is contiguous, split evenly over
 // the grid so the row granularity is 1 and no CTA idles at the end.
-template <int K, int OP, int MAP, int NW, int SR_, int NS_, int F2>
+template <int K, int OP, int MAP, int NW, int SR_, int NS_, int F2, int SM = 1, int LOCK = 0>
 __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel(const __grid_constant__ StreamParams p) {
     constexpr bool TMA = MAP == MAP_TMA;
     constexpr bool HALO = OP != OP_COLS;
@@ -306,6 +325,9 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     while (seg.next(n, s, q0, nrows)) {
         const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
         if (wcol >= p.out_cols) continue;
+        // warps of this strip that have columns (named-barrier thread count for LOCK)
+        const int lock_threads = 32 * min(NW, (p.out_cols - s * (NW * kWarpCols) + kWarpCols - 1) / kWarpCols);
+        (void)lock_threads;
         const int c = wcol + lane * V;                         // this thread's first column
         const int in_row0 = p.row_begin + q0;
         const int steps = nrows + (RING ? K - 1 : 0);
@@ -327,10 +349,10 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             }
         }
 
-        // two copies of the hot loop: the fast store path for warps wholly inside an
-        // image with 8-byte aligned rows, the general one for the ragged edge
-        auto run_chunks = [&](auto fast_tag) {
-        constexpr bool FAST = decltype(fast_tag)::value;
+        // two copies of the hot loop: the fast store path SM and the general one, which
+        // only runs at the ragged right edge (or for rows that are not 8-byte aligned)
+        auto run_chunks = [&](auto mode_tag) {
+        constexpr int SMODE = decltype(mode_tag)::value;
         float acc[RK][V];
 #pragma unroll
         for (int a = 0; a < RK; ++a)
@@ -408,13 +430,18 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                         }
                     }
                     const int q = t - (K - 1);                 // output row completed by this step
-                    oc.put<FAST>(acc[(pr + 1) % K], static_cast<unsigned>(q) < static_cast<unsigned>(nrows), lane);
+                    oc.put<SMODE>(acc[(pr + 1) % K], static_cast<unsigned>(q) < static_cast<unsigned>(nrows), lane);
                 } else {
-                    oc.put<FAST>(b, t < nrows, lane);
+                    oc.put<SMODE>(b, t < nrows, lane);
                 }
             }
             if constexpr (TMA) {
-                __syncwarp();
+                if constexpr (LOCK) {
+                    // CTA lockstep: the active warps of this strip finish the stage together
+                    asm volatile("bar.sync 1, %0;" ::"r"(lock_threads) : "memory");
+                } else {
+                    __syncwarp();
+                }
                 if (lane == 0 && ch + NS < nchunks) {
                     fence_proxy_async_smem();
                     mbar_arrive_expect_tx(&wbar[st], BOX_BYTES);
@@ -423,8 +450,10 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             }
         }
         };
-        if (p.store8 && wcol + kWarpCols <= p.out_cols) run_chunks(std::true_type{});
-        else run_chunks(std::false_type{});
+        // SM (a template parameter) is the store path of warps wholly inside the image; the
+        // host instantiates SM = 2 when every row start is 16-byte aligned, else SM = 1
+        if (wcol + kWarpCols <= p.out_cols && p.store8 >= SM) run_chunks(std::integral_constant<int, SM>{});
+        else run_chunks(std::integral_constant<int, 0>{});
     }
 }
 
@@ -435,11 +464,11 @@ constexpr size_t stream_smem_bytes() {
 }
 
 // The kernel for (K, OP, variant) with the geometry of stream_geom (sepconv_params.h).
-template <int K, int OP, int VARIANT>
+template <int K, int OP, int VARIANT, int SM>
 struct StreamInst {
     static constexpr StreamGeom G = stream_geom(K, OP, VARIANT);
     static constexpr int MAP = VARIANT >= 2 ? MAP_TMA : VARIANT;
-    static constexpr auto kernel = &stream_kernel<K, OP, MAP, G.nw, G.sr, G.ns, G.f2>;
+    static constexpr auto kernel = &stream_kernel<K, OP, MAP, G.nw, G.sr, G.ns, G.f2, SM, G.lock>;
     static constexpr size_t smem = stream_smem_bytes<K, OP, MAP, G.nw, G.sr, G.ns, G.f2>();
     static constexpr int threads = G.nw * 32;
 };

@@ -18,16 +18,17 @@ struct KernelInfo {
     int cps;             // CTAs per SM to size the grid for (0 = occupancy limit)
 };
 
-// streaming kernels: variant = 0 direct, 1 direct 16-byte, 2.. TMA configurations
-// (stream_geom in sepconv_params.h); conv2d: map = MAP_DIRECT / MAP_DIRECT_VEC / MAP_TMA.
-// K in [1, 17]
-KernelInfo stream_rows_info(int map, int K);
-KernelInfo stream_cols_info(int map, int K);
-KernelInfo stream_sep_info(int map, int K);
+// streaming kernels: op = OP_ROWS / OP_COLS / OP_SEP; variant = 0 direct, 1 direct 16-byte,
+// 2.. TMA configurations (stream_geom in sepconv_params.h); smode = 2 if every output row is
+// 16-byte aligned (the 16-byte store path), else 1.  conv2d: map = MAP_DIRECT / _VEC / MAP_TMA.
+// K in [1, 17].
+struct StreamEntry {
+    KernelInfo (*info[2])();
+    cudaError_t (*launch[2])(const StreamParams &, int, cudaStream_t);
+};
+KernelInfo stream_info(int op, int variant, int K, int smode);
+cudaError_t stream_launch(int op, int variant, int K, int smode, const StreamParams &p, int grid, cudaStream_t st);
 KernelInfo conv2d_info(int map, int K);
-cudaError_t stream_rows_launch(int map, int K, const StreamParams &p, int grid, cudaStream_t st);
-cudaError_t stream_cols_launch(int map, int K, const StreamParams &p, int grid, cudaStream_t st);
-cudaError_t stream_sep_launch(int map, int K, const StreamParams &p, int grid, cudaStream_t st);
 cudaError_t conv2d_launch(int map, int K, const Conv2DParams &p, int grid, cudaStream_t st);
 
 // utility kernels (sepconv_util.cu)

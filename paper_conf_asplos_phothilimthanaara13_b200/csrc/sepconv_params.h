@@ -38,7 +38,7 @@ struct alignas(64) StreamParams {
     int nimg;
     int nstrips;                 // CTA strips = ceil(out_cols / (warps*128))
     int parts;                   // >0: row partitions per (image, strip), strided schedule; 0: contiguous
-    int store8;                  // 1: out base, ld_out and image stride give 8-byte aligned rows
+    int store8;                  // 2: every output row 16-byte aligned, 1: 8-byte aligned, 0: neither
     long long total;             // nimg * nstrips * rows (work units)
     float k[kMaxK];
     float2 k2[kMaxK];            // {k_i, k_i}: the same weights as packed-FP32 operands
@@ -65,12 +65,14 @@ struct alignas(64) Conv2DParams {
 // `variant` selects the mapping: 0 direct (4-byte loads), 1 direct (16-byte loads),
 // 2.. the TMA configurations.  The unfused passes have one TMA configuration; the
 // fused kernel has kSepTmaConfigs, all tuner candidates, because the best one moves
-// with K in ways no simple model predicted (e.g. a 6-row, 2-stage ring reaches 97% of
-// a plain copy at K=3 and K=7 while deeper rings lose 8-12%):
-//   cfg 0  8 warps, SR ~ 6 rows (a multiple of K), 2 stages      (shallow)
-//   cfg 1  8 warps, SR ~ 8 rows, up to 3 stages                   (medium)
-//   cfg 2  K <= 9: 16 warps, SR as cfg 0, up to 4 stages;  K >= 10: 8 warps, SR = K,
-//          as many stages as fit (16 warps would spill the K-slot ring at K >= 10)
+// with K in ways no simple model predicts:
+//   cfg 0  SR ~ 6 rows (a multiple of K), 2 stages, CTA lockstep   (shallow)
+//   cfg 1  SR ~ 8 rows, up to 3 stages, CTA lockstep               (medium)
+//   cfg 2  SR ~ 6 rows, 2 stages, warps free-running                (free)
+// "Lockstep" = a CTA barrier after every stage, so the 8 warps of a CTA read the same
+// rows (4 KB of each) together: measured +13% at K=9 and +4% at K=1 on 16384^2, because
+// DRAM sees whole row segments instead of 512-byte pieces at drifting times.  At K=17
+// (FMA-bound) the barrier costs a little, hence cfg 2.
 constexpr int kSepTmaConfigs = 3;
 constexpr int kSmemPerCta = 232448 - 1024;     // opt-in limit minus headroom
 
@@ -82,6 +84,7 @@ SEPCONV_HD constexpr int clampi(int v, int lo, int hi) { return v < lo ? lo : (v
 struct StreamGeom {
     int nw, sr, ns, f2;
     int cps;       // CTAs per SM the grid is sized for (0 = as many as fit)
+    int lock;      // 1: CTA barrier after every stage (TMA only)
 };
 
 SEPCONV_HD constexpr int sep_sr_shallow(int K) { return K >= 6 ? K : K * ((6 + K / 2) / K); }
@@ -90,17 +93,16 @@ SEPCONV_HD constexpr int sep_sr_medium(int K) { return K >= 8 ? K : K * ((8 + K 
 SEPCONV_HD constexpr StreamGeom stream_geom(int K, int op, int variant) {
     // packed FP32 for the column pass: halves its issue slots (FFMA2 peak is ~8% below FFMA's)
     return op == OP_SEP
-               ? (variant < 2 ? StreamGeom{8, K >= 8 ? K : K * ((8 + K - 1) / K), 1, K >= 2 ? 1 : 0, 0}
-                  : variant == 2 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1}
+               ? (variant < 2 ? StreamGeom{8, K >= 8 ? K : K * ((8 + K - 1) / K), 1, K >= 2 ? 1 : 0, 0, 0}
+                  : variant == 2 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1, 1}
                   : variant == 3 ? StreamGeom{8, sep_sr_medium(K),
-                                              clampi(ns_fit(8, sep_sr_medium(K), stream_bw(K, op)), 1, 3), K >= 2 ? 1 : 0, 1}
-                  : K <= 9 ? StreamGeom{16, sep_sr_shallow(K),
-                                        clampi(ns_fit(16, sep_sr_shallow(K), stream_bw(K, op)), 1, 4), K >= 2 ? 1 : 0, 1}
-                           : StreamGeom{8, K, clampi(ns_fit(8, K, stream_bw(K, op)), 1, 8), 1, 1})
-               : op == OP_ROWS ? StreamGeom{8, 8, clampi(ns_fit(8, 8, stream_bw(K, op)), 1, 8), 0, 0}
+                                              clampi(ns_fit(8, sep_sr_medium(K), stream_bw(K, op)), 1, 3), K >= 2 ? 1 : 0,
+                                              1, 1}
+                                 : StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1, 0})
+               : op == OP_ROWS ? StreamGeom{8, 8, clampi(ns_fit(8, 8, stream_bw(K, op)), 1, 8), 0, 0, 0}
                                : StreamGeom{8, K * ((8 + K - 1) / K),
                                             clampi(ns_fit(8, K * ((8 + K - 1) / K), stream_bw(K, op)), 1, 8),
-                                            K >= 2 ? 1 : 0, 0};
+                                            K >= 2 ? 1 : 0, 0, 0};
 }
 SEPCONV_HD constexpr int stream_variants(int op) { return op == OP_SEP ? 2 + kSepTmaConfigs : 3; }
 

@@ -1,5 +1,4 @@
 cd $GRAFT_REPO_ROOT
-for K in 11 13; do
-ncu --set full --clock-control none -k regex:stream_kernel -s 1 -c 1 -o gpurun_out/r01_exp_k$K ./tools/explore 1 $K > gpurun_out/r01_exp_k$K.log 2>&1
-done
-ls -la gpurun_out/
+ncu --set full --clock-control none --import-source on -k regex:stream_kernel -s 1 -c 1 -o gpurun_out/r01_k13_sm1 ./tools/explore 10 13 > gpurun_out/r01_k13_sm1.log 2>&1
+ncu --set full --clock-control none --import-source on -k regex:stream_kernel -s 13 -c 1 -o gpurun_out/r01_k13_sm2 ./tools/explore 10 13 > gpurun_out/r01_k13_sm2.log 2>&1
+ls gpurun_out
