@@ -202,7 +202,8 @@ static int schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int ro
 static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geometry &g, const float *in,
                                          long long ld_in, long long in_img, int in_cols, float *out,
                                          long long ld_out, long long out_img, int out_cols, int rows_total,
-                                         const float *kernel, bool want_tma, int cfg, cudaStream_t st) {
+                                         const float *kernel, bool want_tma, int cfg, int store_path,
+                                         cudaStream_t st) {
     const int K = g.K;
     const bool tma = want_tma && tma_ok(in, ld_in, in_img);
     const bool vec = aligned(in, 16) && (ld_in % 4) == 0 && (in_img % 4) == 0;
@@ -211,7 +212,7 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     const int map = tma ? 2 + std::min(std::max(cfg, 0), ntma - 1) : (vec ? 1 : 0);
     const int store8 = (aligned(out, 16) && (ld_out % 4) == 0 && (out_img % 4) == 0) ? 2
                        : (aligned(out, 8) && (ld_out % 2) == 0 && (out_img % 2) == 0) ? 1 : 0;
-    const int smode = store8 == 2 ? 2 : 1;
+    const int smode = (store8 == 2 && store_path == 0) ? 2 : 1;
     KernelInfo ki = stream_info(op, map, K, smode);
     int occ = 0;
     sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);
@@ -315,7 +316,7 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
     if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st);
     if (c.fused)
         return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, c.config, st);
+                                g.out_cols, g.rows, kernel, tma, c.config, c.store, st);
     // Choice 2 as the paper writes it: ConvolveRows into buffer, then ConvolveColumns.
     // The buffer holds the rows this launch's output rows need: [row_begin, row_begin + rows + K - 1).
     if (!buf) return fail(SEPCONV_E_INVALID, "unfused separable needs a workspace");
@@ -333,7 +334,7 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
         gg.in_rows = g.in_rows - g.row_begin;
         gg.row_begin = 0;
         sepconv_status_t s = launch_stream_op(plan, OP_ROWS, gg, in0, g.ld_in, g.in_img, g.in_cols, buf, ld_buf,
-                                              buf_img, g.out_cols, brows, kernel, tma, 0, st);
+                                              buf_img, g.out_cols, brows, kernel, tma, 0, 0, st);
         if (s != SEPCONV_OK) return s;
     }
     {
@@ -342,15 +343,15 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
         gc.row_begin = 0;
         float *out0 = out + static_cast<long long>(g.row_begin) * g.ld_out;
         return launch_stream_op(plan, OP_COLS, gc, buf, ld_buf, buf_img, g.out_cols, out0, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, 0, st);
+                                g.out_cols, g.rows, kernel, tma, 0, 0, st);
     }
 }
 
 // Static default before tuning (R16): fused separable with TMA for K >= 2
 // (one HBM pass, 2K FMA/px), 2D with TMA for K = 1.
 static Candidate default_candidate(int K, sepconv_variant_t v) {
-    if (v == SEPCONV_2D || (v == SEPCONV_AUTO && K == 1)) return {SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0};
-    return {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, 0};
+    if (v == SEPCONV_2D || (v == SEPCONV_AUTO && K == 1)) return {SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0, 0};
+    return {SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, 0, 0};
 }
 
 int candidate_warps(int K, const Candidate &c) {
@@ -363,7 +364,7 @@ Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v) {
     const int idx = v == SEPCONV_2D ? 0 : v == SEPCONV_SEPARABLE ? 1 : 2;
     if (plan->tuned) {
         const sepconv_choice_t &c = plan->best[idx];
-        return {static_cast<int>(c.algo), c.mapping, c.fused, c.config};
+        return {static_cast<int>(c.algo), c.mapping, c.fused, c.config, c.store_path};
     }
     return default_candidate(plan->k, v);
 }
@@ -503,6 +504,7 @@ static sepconv_status_t check_choice(const sepconv_choice_t *c) {
         return fail(SEPCONV_E_INVALID, "choice.mapping must be DIRECT or TMA");
     if (c->config < 0 || c->config >= kSepTmaConfigs)
         return fail(SEPCONV_E_INVALID, "choice.config must be in [0, %d)", kSepTmaConfigs);
+    if (c->store_path < 0 || c->store_path > 1) return fail(SEPCONV_E_INVALID, "choice.store_path must be 0 or 1");
     return SEPCONV_OK;
 }
 
@@ -541,7 +543,7 @@ sepconv_status_t sepconv_run_choice(sepconv_plan_t plan, const float *in, const 
     sepconv_status_t s = check_choice(choice);
     if (s != SEPCONV_OK) return s;
     Candidate c{static_cast<int>(choice->algo), choice->mapping, choice->algo == SEPCONV_SEPARABLE ? choice->fused : 0,
-                choice->config};
+                choice->config, choice->store_path};
     return run_resolved(plan, in, kernel, out, c, static_cast<cudaStream_t>(stream));
 }
 
@@ -560,6 +562,7 @@ sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t varia
         choice->mapping = c.mapping;
         choice->fused = c.fused;
         choice->config = c.config;
+        choice->store_path = c.store;
         choice->warps = candidate_warps(plan->k, c);
         choice->ctas_per_sm = 1;
     }

@@ -14,6 +14,7 @@ const StreamEntry *stream_table_sep_v1();
 const StreamEntry *stream_table_sep_v2();
 const StreamEntry *stream_table_sep_v3();
 const StreamEntry *stream_table_sep_v4();
+const StreamEntry *stream_table_sep_v5();
 
 static const StreamEntry *table(int op, int variant) {
     switch (op) {
@@ -38,6 +39,7 @@ static const StreamEntry *table(int op, int variant) {
                 case 2: return stream_table_sep_v2();
                 case 3: return stream_table_sep_v3();
                 case 4: return stream_table_sep_v4();
+                case 5: return stream_table_sep_v5();
             }
             break;
     }

@@ -45,6 +45,7 @@ struct Candidate {
     int mapping;   // SEPCONV_MAP_DIRECT / SEPCONV_MAP_TMA
     int fused;     // separable only
     int config;    // fused + TMA: stage configuration 0..kSepTmaConfigs-1 (stream_geom)
+    int store;     // 0: 16-byte store path when every output row allows it, 1: always the 8-byte path
 };
 
 struct TensorMapCache {

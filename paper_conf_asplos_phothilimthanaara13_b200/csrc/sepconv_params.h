@@ -66,14 +66,16 @@ struct alignas(64) Conv2DParams {
 // 2.. the TMA configurations.  The unfused passes have one TMA configuration; the
 // fused kernel has kSepTmaConfigs, all tuner candidates, because the best one moves
 // with K in ways no simple model predicts:
-//   cfg 0  SR ~ 6 rows (a multiple of K), 2 stages, CTA lockstep   (shallow)
-//   cfg 1  SR ~ 8 rows, up to 3 stages, CTA lockstep               (medium)
-//   cfg 2  SR ~ 6 rows, 2 stages, warps free-running                (free)
+//   cfg 0  8 warps, SR ~ 6 rows (a multiple of K), 2 stages, CTA lockstep   (shallow)
+//   cfg 1  8 warps, SR ~ 8 rows, up to 3 stages, CTA lockstep               (medium)
+//   cfg 2  8 warps, SR ~ 6 rows, 2 stages, warps free-running                (free)
+//   cfg 3  16 warps, SR ~ 6 rows, as many stages as fit (<= 4), free-running (wide)
 // "Lockstep" = a CTA barrier after every stage, so the 8 warps of a CTA read the same
 // rows (4 KB of each) together: measured +13% at K=9 and +4% at K=1 on 16384^2, because
 // DRAM sees whole row segments instead of 512-byte pieces at drifting times.  At K=17
-// (FMA-bound) the barrier costs a little, hence cfg 2.
-constexpr int kSepTmaConfigs = 3;
+// (FMA-bound) the barrier costs a little, hence cfg 2; and there 16 warps (cfg 3, 128
+// registers, a few spilled) beat 8 warps with 2 stages by 10%.
+constexpr int kSepTmaConfigs = 4;
 constexpr int kSmemPerCta = 232448 - 1024;     // opt-in limit minus headroom
 
 SEPCONV_HD constexpr int stream_bw(int K, int op) { return 32 * 4 + (op != OP_COLS ? (((K - 1) + 3) & ~3) : 0); }
@@ -98,7 +100,10 @@ SEPCONV_HD constexpr StreamGeom stream_geom(int K, int op, int variant) {
                   : variant == 3 ? StreamGeom{8, sep_sr_medium(K),
                                               clampi(ns_fit(8, sep_sr_medium(K), stream_bw(K, op)), 1, 3), K >= 2 ? 1 : 0,
                                               1, 1}
-                                 : StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1, 0})
+                  : variant == 4 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1, 0}
+                                 : StreamGeom{16, sep_sr_shallow(K),
+                                              clampi(ns_fit(16, sep_sr_shallow(K), stream_bw(K, op)), 1, 4),
+                                              K >= 2 ? 1 : 0, 1, 0})
                : op == OP_ROWS ? StreamGeom{8, 8, clampi(ns_fit(8, 8, stream_bw(K, op)), 1, 8), 0, 0, 0}
                                : StreamGeom{8, K * ((8 + K - 1) / K),
                                             clampi(ns_fit(8, K * ((8 + K - 1) / K), stream_bw(K, op)), 1, 8),

@@ -25,15 +25,20 @@ using namespace sepconv;
 
 namespace {
 
-std::vector<Candidate> candidates(sepconv_plan_t) {
+std::vector<Candidate> candidates(sepconv_plan_t p) {
     // fixed order: this is also the tie-break order
     std::vector<Candidate> cs;
-    for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg});
-    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1, 0});
-    cs.push_back({SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0});
-    cs.push_back({SEPCONV_2D, SEPCONV_MAP_DIRECT, 0, 0});
-    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 0, 0});
-    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 0, 0});
+    for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 0});
+    // with 16-byte aligned output rows the 8-byte store path is a distinct candidate
+    // (it paces the warps differently; measured faster at K=13 on 16384^2)
+    const bool rows16 = (p->ld_out % 4) == 0;
+    if (rows16)
+        for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 1});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1, 0, 0});
+    cs.push_back({SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0, 0});
+    cs.push_back({SEPCONV_2D, SEPCONV_MAP_DIRECT, 0, 0, 0});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 0, 0, 0});
+    cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 0, 0, 0});
     return cs;
 }
 
@@ -48,8 +53,8 @@ std::string cache_key(sepconv_plan_t p) {
 
 std::string choice_json(const sepconv_choice_t &c) {
     char b[160];
-    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%.9g]", (int)c.algo, c.mapping, c.fused, c.config, c.warps,
-             c.ctas_per_sm, c.median_us);
+    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g]", (int)c.algo, c.mapping, c.fused, c.config, c.store_path,
+             c.warps, c.ctas_per_sm, c.median_us);
     return b;
 }
 
@@ -57,17 +62,19 @@ bool parse_choice(const std::string &line, const char *field, sepconv_choice_t *
     std::string f = std::string("\"") + field + "\":[";
     size_t pos = line.find(f);
     if (pos == std::string::npos) return false;
-    int algo, map, fused, config, warps, ctas;
+    int algo, map, fused, config, store, warps, ctas;
     float us;
-    if (sscanf(line.c_str() + pos + f.size(), "%d,%d,%d,%d,%d,%d,%f", &algo, &map, &fused, &config, &warps, &ctas,
-               &us) != 7)
+    if (sscanf(line.c_str() + pos + f.size(), "%d,%d,%d,%d,%d,%d,%d,%f", &algo, &map, &fused, &config, &store, &warps,
+               &ctas, &us) != 8)
         return false;
+    if (store < 0 || store > 1) return false;
     if (config < 0 || config >= kSepTmaConfigs) return false;
     if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return false;
     c->algo = static_cast<sepconv_variant_t>(algo);
     c->mapping = map;
     c->fused = fused;
     c->config = config;
+    c->store_path = store;
     c->warps = warps;
     c->ctas_per_sm = ctas;
     c->median_us = us;
@@ -126,6 +133,7 @@ sepconv_status_t sepconv_get_candidate(sepconv_plan_t plan, int index, sepconv_c
     choice->mapping = cs[index].mapping;
     choice->fused = cs[index].fused;
     choice->config = cs[index].config;
+    choice->store_path = cs[index].store;
     choice->warps = candidate_warps(plan->k, cs[index]);
     choice->ctas_per_sm = 1;
     return SEPCONV_OK;
@@ -242,6 +250,7 @@ sepconv_status_t sepconv_tune(sepconv_plan_t plan, const sepconv_tune_opts_t *op
         o.mapping = c.mapping;
         o.fused = c.fused;
         o.config = c.config;
+        o.store_path = c.store;
         o.warps = candidate_warps(plan->k, c);
         o.ctas_per_sm = 1;
         o.median_us = med[bi[s]];

@@ -45,7 +45,8 @@ class _Desc(ctypes.Structure):
 
 class _Choice(ctypes.Structure):
     _fields_ = [("algo", ctypes.c_int), ("mapping", ctypes.c_int), ("fused", ctypes.c_int),
-                ("config", ctypes.c_int), ("warps", ctypes.c_int), ("ctas_per_sm", ctypes.c_int),
+                ("config", ctypes.c_int), ("store_path", ctypes.c_int), ("warps", ctypes.c_int),
+                ("ctas_per_sm", ctypes.c_int),
                 ("median_us", ctypes.c_float)]
 
 
@@ -59,6 +60,7 @@ class Choice:
     mapping: int
     fused: int
     config: int = 0
+    store_path: int = 0
     warps: int = 8
     ctas_per_sm: int = 1
     median_us: float = 0.0
@@ -68,18 +70,19 @@ class Choice:
         a = "2d" if self.algo == SEPCONV_2D else ("sep-fused" if self.fused else "sep-unfused")
         m = ("-tma" if self.mapping == MAP_TMA else "-direct")
         if self.algo == SEPCONV_SEPARABLE and self.fused and self.mapping == MAP_TMA:
-            m += "%d" % self.config
+            m += "%d" % self.config + ("s8" if self.store_path else "")
         return a + m
 
     def key(self):
-        return (self.algo, self.mapping, self.fused, self.config)
+        return (self.algo, self.mapping, self.fused, self.config, self.store_path)
 
     def _c(self) -> _Choice:
-        return _Choice(self.algo, self.mapping, self.fused, self.config, self.warps, self.ctas_per_sm, self.median_us)
+        return _Choice(self.algo, self.mapping, self.fused, self.config, self.store_path, self.warps, self.ctas_per_sm,
+                       self.median_us)
 
     @staticmethod
     def _from(c: _Choice) -> "Choice":
-        return Choice(c.algo, c.mapping, c.fused, c.config, c.warps, c.ctas_per_sm, float(c.median_us))
+        return Choice(c.algo, c.mapping, c.fused, c.config, c.store_path, c.warps, c.ctas_per_sm, float(c.median_us))
 
 
 _lib = None

@@ -19,6 +19,8 @@ CANDS = [
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 0),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 1),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 3),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 0, 1),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_DIRECT, 1),
     sc.Choice(sc.SEPCONV_2D, sc.MAP_TMA, 0),
     sc.Choice(sc.SEPCONV_2D, sc.MAP_DIRECT, 0),
@@ -209,7 +211,7 @@ def test_errors():
 def test_launch_count_increases():
     before = sc.launch_count()
     img = synth.uniform_image(64, 300, seed=1)
-    run_gpu(img, synth.binomial_kernel(5), CANDS[6])          # unfused: 2 launches
+    run_gpu(img, synth.binomial_kernel(5), CANDS[8])          # unfused: 2 launches
     assert sc.launch_count() == before + 2
 
 

@@ -49,10 +49,10 @@ static float time_it_(F f, int reps) {
     return t[t.size() / 2];
 }
 
-template <int K, int OP, int MAP, int NW, int SR, int NS, int F2 = 0, int SM = 1>
+template <int K, int OP, int MAP, int NW, int SR, int NS, int F2 = 0, int SM = 1, int LOCK = 0>
 static void run_cfg(int ctas_per_sm, CUtensorMapL2promotion prom, const char *tag, int parts = 0) {
     if (g_onlyK && g_onlyK != K) return;
-    auto kern = stream_kernel<K, OP, MAP, NW, SR, NS, F2, SM>;
+    auto kern = stream_kernel<K, OP, MAP, NW, SR, NS, F2, SM, LOCK>;
     size_t smem = stream_smem_bytes<K, OP, MAP, NW, SR, NS, F2>();
     if (MAP == MAP_TMA && NW * NS * (((SR * stream_bw(K, OP) + 31) & ~31) * 4 + 8) > kSmemPerCta) { printf("skip\n"); return; }
     if (smem > 232448) { printf("skip (smem %zu)\n", smem); return; }
@@ -88,7 +88,7 @@ static void run_cfg(int ctas_per_sm, CUtensorMapL2promotion prom, const char *ta
     float us = time_it([&] { kern<<<grid, NW * 32, smem>>>(p); });
     cudaError_t e = cudaGetLastError();
     double bytes = 4.0 * ((double)H * W + (double)(H - K + 1) * (W - K + 1));
-    printf("K=%2d SM=%d F2=%d %-6s map=%d NW=%2d SR=%2d NS=%d cps=%d/%d prom=%d parts=%d grid=%d smem=%3zuKB : %7.1f us  %6.0f GB/s %s\n", K, SM, F2, tag, MAP, NW,
+    printf("K=%2d L=%d SM=%d F2=%d %-6s map=%d NW=%2d SR=%2d NS=%d cps=%d/%d prom=%d parts=%d grid=%d smem=%3zuKB : %7.1f us  %6.0f GB/s %s\n", K, LOCK, SM, F2, tag, MAP, NW,
            SR, NS, cps, occ, (int)prom, parts, grid, smem / 1024, us, bytes / us / 1e3, e ? cudaGetErrorString(e) : "");
 }
 
@@ -114,17 +114,14 @@ int main(int argc, char **argv) {
     }
     const auto P0 = CU_TENSOR_MAP_L2_PROMOTION_NONE, P256 = CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                P128 = CU_TENSOR_MAP_L2_PROMOTION_L2_128B;
-    run_cfg<13, OP_SEP, MAP_TMA, 8, 13, 3, 1, 1>(1, P0, "sm", -1);
-    run_cfg<13, OP_SEP, MAP_TMA, 8, 13, 3, 1, 2>(1, P0, "sm", -1);
-    run_cfg<13, OP_SEP, MAP_TMA, 8, 13, 2, 1, 1>(1, P0, "sm", -1);
-    run_cfg<13, OP_SEP, MAP_TMA, 8, 13, 2, 1, 2>(1, P0, "sm", -1);
-    run_cfg<17, OP_SEP, MAP_TMA, 8, 17, 2, 1, 1>(1, P0, "sm", -1);
-    run_cfg<17, OP_SEP, MAP_TMA, 8, 17, 2, 1, 2>(1, P0, "sm", -1);
-    run_cfg<9, OP_SEP, MAP_TMA, 8, 9, 2, 1, 1>(1, P0, "sm", -1);
-    run_cfg<9, OP_SEP, MAP_TMA, 8, 9, 2, 1, 2>(1, P0, "sm", -1);
-    run_cfg<5, OP_SEP, MAP_TMA, 8, 5, 2, 1, 1>(1, P0, "sm", -1);
-    run_cfg<5, OP_SEP, MAP_TMA, 8, 5, 2, 1, 2>(1, P0, "sm", -1);
-    run_cfg<1, OP_SEP, MAP_TMA, 8, 6, 2, 0, 1>(1, P0, "sm", -1);
-    run_cfg<1, OP_SEP, MAP_TMA, 8, 6, 2, 0, 2>(1, P0, "sm", -1);
+    run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 2, 0>(1, P0, "x", -1);
+    run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 2, 1>(1, P0, "x", -1);
+    run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<15, OP_SEP, MAP_TMA, 16, 15, 1, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<15, OP_SEP, MAP_TMA, 16, 15, 1, 1, 1, 1>(1, P0, "x", -1);
+    run_cfg<13, OP_SEP, MAP_TMA, 16, 13, 1, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<13, OP_SEP, MAP_TMA, 16, 13, 1, 1, 2, 0>(1, P0, "x", -1);
+    run_cfg<11, OP_SEP, MAP_TMA, 16, 11, 2, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<11, OP_SEP, MAP_TMA, 16, 11, 1, 1, 1, 0>(1, P0, "x", -1);
     return 0;
 }
