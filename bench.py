@@ -146,8 +146,8 @@ def oracle_sample(img_rows_fn, W, widths, target_s, nthreads=0):
             px += out.size
         return time.perf_counter() - t0, px
 
-    t_probe, _ = run(4)
-    S = int(max(4, min(4096, 4 * target_s / max(t_probe, 1e-4))))
+    t_probe, _ = run(16)
+    S = int(max(16, min(8192, 16 * target_s / max(t_probe, 1e-4))))
     t, px = run(S)
     return {"value": px / t / 1e6, "unit": "Mpixels/s", "cores": cores, "kind": "oracle",
             "sample": f"first {S} output rows x {W - min(widths) + 1}..{W - kmax + 1} cols of the image, "
@@ -301,6 +301,7 @@ def main():
         torch.cuda.synchronize()
         if dist:
             dist.barrier()
+        torch.cuda.nvtx.range_push("sepconv_timed")      # ncu --nvtx-include sepconv_timed/
         e_start.record(stream)
         for s in range(args.steps):
             for K in widths:
@@ -308,10 +309,15 @@ def main():
                 one_pass(K)
                 ev[K][s][1].record(stream)
         e_end.record(stream)
+        torch.cuda.nvtx.range_pop()
         torch.cuda.synchronize()
         if dist:
             dist.barrier()
     launches = sc.launch_count() - launches0
+    if dist:
+        tl = torch.tensor([launches], dtype=torch.int64, device=dev)
+        dist.all_reduce(tl)
+        launches = int(tl.item())
     total_ms = e_start.elapsed_time(e_end)
     per_k_ms = {K: sum(a.elapsed_time(b) for a, b in ev[K]) / args.steps for K in widths}
     if dist:

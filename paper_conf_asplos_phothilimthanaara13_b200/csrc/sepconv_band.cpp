@@ -91,6 +91,7 @@ void sepconv_comm_destroy_internal(sepconv_plan_t plan) {
     if (plan->ev_halo) cudaEventDestroy(plan->ev_halo);
     plan->comm_stream = nullptr;
     plan->ev_in = plan->ev_halo = nullptr;
+    plan->band_external = false;
 }
 
 extern "C" {
@@ -127,11 +128,9 @@ sepconv_status_t sepconv_nccl_unique_id(unsigned char id[SEPCONV_NCCL_ID_BYTES])
 
 sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[SEPCONV_NCCL_ID_BYTES], int nranks,
                                    int rank) {
-    if (!plan || !id) return fail(SEPCONV_E_INVALID, "NULL argument");
+    if (!plan) return fail(SEPCONV_E_INVALID, "NULL plan");
     if (nranks < 1 || rank < 0 || rank >= nranks) return fail(SEPCONV_E_INVALID, "rank %d of %d", rank, nranks);
     if (plan->n != 1) return fail(SEPCONV_E_INVALID, "row bands split a single image (plan has n=%lld)", (long long)plan->n);
-    NcclApi &a = nccl();
-    if (!a.ok) return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
     int prev = -1;
     cudaGetDevice(&prev);
     SC_CUDA(cudaSetDevice(plan->dev.device));
@@ -139,6 +138,19 @@ sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[S
     SC_CUDA(cudaStreamCreateWithFlags(&plan->comm_stream, cudaStreamNonBlocking));
     SC_CUDA(cudaEventCreateWithFlags(&plan->ev_in, cudaEventDisableTiming));
     SC_CUDA(cudaEventCreateWithFlags(&plan->ev_halo, cudaEventDisableTiming));
+    plan->nranks = nranks;
+    plan->rank = rank;
+    if (!id) {                        // external-halo mode: the caller moves the halo rows
+        plan->band_external = true;
+        if (prev >= 0) cudaSetDevice(prev);
+        return SEPCONV_OK;
+    }
+    plan->band_external = false;
+    NcclApi &a = nccl();
+    if (!a.ok) {
+        if (prev >= 0) cudaSetDevice(prev);
+        return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
+    }
     nccl_unique_id_t u;
     std::memcpy(u.internal, id, SEPCONV_NCCL_ID_BYTES);
     nccl_comm_t comm = nullptr;
@@ -146,15 +158,14 @@ sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[S
     if (prev >= 0) cudaSetDevice(prev);
     if (r != 0) return nccl_fail(r, "ncclCommInitRank");
     plan->comm = comm;
-    plan->nranks = nranks;
-    plan->rank = rank;
     return SEPCONV_OK;
 }
 
 sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const float *kernel, float *out_band,
                                   sepconv_variant_t variant, sepconv_stream_t stream) {
     if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
-    if (!plan->comm) return fail(SEPCONV_E_INVALID, "sepconv_comm_init has not been called on this plan");
+    if (!plan->comm && !plan->band_external)
+        return fail(SEPCONV_E_INVALID, "sepconv_comm_init has not been called on this plan");
     if (!in_band || !out_band) return fail(SEPCONV_E_INVALID, "NULL band pointer");
     if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
         return fail(SEPCONV_E_INVALID, "bad variant");
@@ -180,7 +191,7 @@ sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const flo
     // 1. the exchange (comm stream, after the caller's writes to in_band on `st`)
     SC_CUDA(cudaEventRecord(plan->ev_in, st));
     SC_CUDA(cudaStreamWaitEvent(plan->comm_stream, plan->ev_in, 0));
-    if (halo > 0 && plan->nranks > 1) {
+    if (halo > 0 && plan->nranks > 1 && !plan->band_external) {
         const size_t cnt = static_cast<size_t>(halo) * plan->ld_in;
         nccl_comm_t comm = static_cast<nccl_comm_t>(plan->comm);
         nccl_result_t r = a.GroupStart();

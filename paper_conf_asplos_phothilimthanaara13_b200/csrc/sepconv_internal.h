@@ -83,6 +83,7 @@ struct sepconv_plan_s {
 
     // NCCL (row bands)
     void *comm = nullptr;
+    bool band_external = false;   // sepconv_comm_init(id = NULL): the caller supplies the halo rows
     int nranks = 1, rank = 0;
     cudaStream_t comm_stream = nullptr;
     cudaEvent_t ev_in = nullptr, ev_halo = nullptr;

@@ -284,8 +284,9 @@ class Plan:
         return res
 
     # -- row bands --
-    def comm_init(self, unique_id: bytes, nranks: int, rank: int):
-        if len(unique_id) != NCCL_ID_BYTES:
+    def comm_init(self, unique_id: bytes | None, nranks: int, rank: int):
+        """NCCL communicator for row bands; unique_id=None = external-halo mode (caller moves halos)."""
+        if unique_id is not None and len(unique_id) != NCCL_ID_BYTES:
             raise ValueError("NCCL unique id must be 128 bytes")
         _check(lib().sepconv_comm_init(self._h, unique_id, int(nranks), int(rank)), "sepconv_comm_init")
 

@@ -1,0 +1,61 @@
+"""The paper's Fig. 2 re-run on B200: execution time of every mapping of
+SeparableConvolution vs kernel width, plus the tuner's pick.
+
+    python tools/fig2.py [--size 3520] [--widths 3,5,...,17] [--reps 20] > profiles/r01_fig2_3520.json
+
+Mappings (the paper's four: 2D / Separable x local memory / no local memory)
+are the C ABI's candidates: 2d-direct, 2d-tma, sep-unfused-direct, sep-unfused-tma, plus
+the B200-only fused separable kernels (sep-fused-*).  Times are device times (CUDA events,
+median of --reps, L2 flushed before each run when the working set fits in L2); the paper's
+include PCIe copies, so only the shape of the curves is comparable.
+"""
+import argparse
+import json
+import os
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+import torch  # noqa: E402
+
+from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc  # noqa: E402
+from paper_conf_asplos_phothilimthanaara13_b200 import synth  # noqa: E402
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--size", type=int, default=3520)
+    ap.add_argument("--widths", default="3,5,7,9,11,13,15,17")
+    ap.add_argument("--reps", type=int, default=20)
+    a = ap.parse_args()
+    H = W = a.size
+    img = torch.from_numpy(synth.uniform_image(H, W, seed=synth.BENCH_SEED_BASE + 2)).cuda()
+    flush = torch.empty(int(torch.cuda.get_device_properties(0).L2_cache_size // 2), device="cuda")
+    res = {"size": [H, W], "widths": {}, "unit": "us", "timing": "median of %d, L2 flushed" % a.reps}
+    for K in [int(x) for x in a.widths.split(",")]:
+        k = synth.binomial_kernel(K)
+        p = sc.Plan(H, W, K)
+        out = torch.empty((H - K + 1, W - K + 1), device="cuda")
+        row = {}
+        for c in p.candidates():
+            ts = []
+            for r in range(a.reps + 3):
+                flush.zero_()
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record()
+                p.run_choice(img, k, out, c)
+                e1.record()
+                torch.cuda.synchronize()
+                if r >= 3:
+                    ts.append(e0.elapsed_time(e1) * 1e3)
+            ts.sort()
+            row[c.name] = ts[len(ts) // 2]
+        best = p.tune(reps=a.reps)
+        row["tuner"] = {"pick": best.name, "us": best.median_us}
+        res["widths"][str(K)] = row
+        print(K, {n: round(v, 1) for n, v in row.items() if n != "tuner"}, row["tuner"], file=sys.stderr)
+    print(json.dumps(res))
+
+
+if __name__ == "__main__":
+    main()
