@@ -175,12 +175,31 @@ struct OutCursor {
             : "memory");
         ptr += ld;
     }
-    // MODE 2: 16-byte rows, 1: 8-byte rows, 0: general (ragged edge, 4-byte rows)
+    // Ragged right edge / 4-byte aligned rows of the streaming kernels: per-element
+    // predicated 4-byte stores only (cheap in registers: this body is compiled next to the
+    // hot one and the kernel's register budget is the larger of the two).
+    __device__ __forceinline__ void store_scalar(const float (&v)[V], bool ok) {
+        const unsigned q0 = ok && e0, q1 = ok && e1, q2 = ok && e2, q3 = ok && e3;
+        asm volatile(
+            "{\n\t.reg .pred q0, q1, q2, q3;\n\t"
+            "setp.ne.u32 q0, %5, 0;\n\t"
+            "setp.ne.u32 q1, %6, 0;\n\t"
+            "setp.ne.u32 q2, %7, 0;\n\t"
+            "setp.ne.u32 q3, %8, 0;\n\t"
+            "@q0 st.global.f32 [%0], %1;\n\t"
+            "@q1 st.global.f32 [%0+4], %2;\n\t"
+            "@q2 st.global.f32 [%0+8], %3;\n\t"
+            "@q3 st.global.f32 [%0+12], %4;\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(q0), "r"(q1), "r"(q2), "r"(q3)
+            : "memory");
+        ptr += ld;
+    }
+    // MODE 2: 16-byte rows, 1: 8-byte rows, 0: ragged edge / 4-byte rows
     template <int MODE>
     __device__ __forceinline__ void put(const float (&v)[V], bool ok, int lane) {
         if constexpr (MODE == 2) store_fast16(v, ok);
         else if constexpr (MODE == 1) store_fast(v, ok, lane);
-        else store(v, ok);
+        else store_scalar(v, ok);
     }
     // write v to the cursor row if ok, then move to the next row
     __device__ __forceinline__ void store(const float (&v)[V], bool ok) {

@@ -115,13 +115,16 @@ int main(int argc, char **argv) {
     const auto P0 = CU_TENSOR_MAP_L2_PROMOTION_NONE, P256 = CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                P128 = CU_TENSOR_MAP_L2_PROMOTION_L2_128B;
     run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 2, 0>(1, P0, "x", -1);
-    run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 2, 1>(1, P0, "x", -1);
-    run_cfg<17, OP_SEP, MAP_TMA, 16, 17, 1, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<17, OP_SEP, MAP_TMA, 8, 17, 2, 1, 2, 0>(1, P0, "x", -1);
     run_cfg<15, OP_SEP, MAP_TMA, 16, 15, 1, 1, 1, 0>(1, P0, "x", -1);
-    run_cfg<15, OP_SEP, MAP_TMA, 16, 15, 1, 1, 1, 1>(1, P0, "x", -1);
+    run_cfg<15, OP_SEP, MAP_TMA, 8, 15, 2, 1, 1, 0>(1, P0, "x", -1);
     run_cfg<13, OP_SEP, MAP_TMA, 16, 13, 1, 1, 1, 0>(1, P0, "x", -1);
-    run_cfg<13, OP_SEP, MAP_TMA, 16, 13, 1, 1, 2, 0>(1, P0, "x", -1);
-    run_cfg<11, OP_SEP, MAP_TMA, 16, 11, 2, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<13, OP_SEP, MAP_TMA, 8, 13, 3, 1, 1, 0>(1, P0, "x", -1);
     run_cfg<11, OP_SEP, MAP_TMA, 16, 11, 1, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<11, OP_SEP, MAP_TMA, 8, 11, 2, 1, 1, 1>(1, P0, "x", -1);
+    run_cfg<9, OP_SEP, MAP_TMA, 8, 9, 2, 1, 2, 1>(1, P0, "x", -1);
+    run_cfg<3, OP_SEP, MAP_TMA, 8, 6, 2, 1, 1, 0>(1, P0, "x", -1);
+    run_cfg<5, OP_SEP, MAP_TMA, 8, 5, 2, 1, 2, 0>(1, P0, "x", -1);
+    run_cfg<7, OP_SEP, MAP_TMA, 8, 7, 2, 1, 1, 0>(1, P0, "x", -1);
     return 0;
 }
