@@ -242,7 +242,7 @@ def main():
         plans, outs, ins = {}, {}, {}
         for K in widths:
             r0, rows, owned, alloc = bands[K]
-            p = sc.Plan(alloc, W, K)
+            p = sc.Plan(alloc, W, K, device=local)
             if world > 1:
                 uid = sc.nccl_unique_id() if rank == 0 else bytes(sc.NCCL_ID_BYTES)
                 t = torch.tensor(list(uid), dtype=torch.uint8, device=dev)
@@ -263,7 +263,7 @@ def main():
         host_img = np.stack([synth.uniform_image(H, W, seed, n=n0 + i) for i in range(per)])
         dev_img = torch.from_numpy(host_img).to(dev)
         K = widths[0]
-        plans = {K: sc.Plan(H, W, K, n=per)}
+        plans = {K: sc.Plan(H, W, K, n=per, device=local)}
         outs = {K: torch.empty((per, H - K + 1, W - K + 1), dtype=torch.float32, device=dev)}
         ins = {K: dev_img}
         out_px_rank = {K: outs[K].numel()}
@@ -379,7 +379,7 @@ def main():
             h_in = torch.from_numpy(host_img).pin_memory()
             for K in widths:
                 r0, rows, owned, alloc = bands[K]
-                hplans[K] = sc.Plan(alloc, W, K)
+                hplans[K] = sc.Plan(alloc, W, K, device=local)
                 hplans[K].tune(reps=3)
                 h_out[K] = torch.empty((rows, W - K + 1), dtype=torch.float32).pin_memory()
         else:
