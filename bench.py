@@ -240,14 +240,17 @@ def main():
         dev_img = torch.empty((r_hi - r_lo + kmax, W), dtype=torch.float32, device=dev)
         dev_img[:host_img.shape[0]].copy_(torch.from_numpy(host_img))
         plans, outs, ins = {}, {}, {}
+        uid = None
+        if world > 1:                                   # one NCCL communicator shared by every width's plan
+            raw = sc.nccl_unique_id() if rank == 0 else bytes(sc.NCCL_ID_BYTES)
+            t = torch.tensor(list(raw), dtype=torch.uint8, device=dev)
+            dist.broadcast(t, 0)
+            uid = bytes(t.cpu().tolist())
         for K in widths:
             r0, rows, owned, alloc = bands[K]
             p = sc.Plan(alloc, W, K, device=local)
             if world > 1:
-                uid = sc.nccl_unique_id() if rank == 0 else bytes(sc.NCCL_ID_BYTES)
-                t = torch.tensor(list(uid), dtype=torch.uint8, device=dev)
-                dist.broadcast(t, 0)
-                p.comm_init(bytes(t.cpu().tolist()), world, rank)
+                p.comm_init(uid, world, rank)
             plans[K] = p
             outs[K] = torch.empty((rows, W - K + 1), dtype=torch.float32, device=dev)
             # the band's own input rows; rows past `owned` are the halo, written by run_band

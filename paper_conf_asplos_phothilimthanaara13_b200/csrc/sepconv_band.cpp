@@ -14,7 +14,9 @@
 
 #include <cstdlib>
 #include <cstring>
+#include <map>
 #include <mutex>
+#include <string>
 
 #include "sepconv_internal.h"
 
@@ -76,6 +78,29 @@ NcclApi &nccl() {
     return api;
 }
 
+// Communicators are shared by every plan of the process that is initialised with the same
+// unique id, rank and size (e.g. one plan per kernel width over the same row bands): the
+// first sepconv_comm_init creates it collectively, later ones take a reference.
+struct SharedComm {
+    nccl_comm_t comm = nullptr;
+    int nranks = 0, rank = 0, refs = 0, device = -1;
+};
+std::mutex g_comm_mu;
+std::map<std::string, SharedComm> g_comms;
+
+void release_comm(void *comm) {
+    std::lock_guard<std::mutex> lock(g_comm_mu);
+    for (auto it = g_comms.begin(); it != g_comms.end(); ++it) {
+        if (it->second.comm == comm) {
+            if (--it->second.refs == 0) {
+                if (nccl().ok) nccl().CommDestroy(it->second.comm);
+                g_comms.erase(it);
+            }
+            return;
+        }
+    }
+}
+
 sepconv_status_t nccl_fail(nccl_result_t r, const char *what) {
     NcclApi &a = nccl();
     return fail(SEPCONV_E_NCCL, "%s: %s", what, a.GetErrorString ? a.GetErrorString(r) : "error");
@@ -84,7 +109,7 @@ sepconv_status_t nccl_fail(nccl_result_t r, const char *what) {
 }  // namespace
 
 void sepconv_comm_destroy_internal(sepconv_plan_t plan) {
-    if (plan->comm && nccl().ok) nccl().CommDestroy(static_cast<nccl_comm_t>(plan->comm));
+    if (plan->comm) release_comm(plan->comm);
     plan->comm = nullptr;
     if (plan->comm_stream) cudaStreamDestroy(plan->comm_stream);
     if (plan->ev_in) cudaEventDestroy(plan->ev_in);
@@ -151,12 +176,32 @@ sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[S
         if (prev >= 0) cudaSetDevice(prev);
         return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
     }
+    const std::string key(reinterpret_cast<const char *>(id), SEPCONV_NCCL_ID_BYTES);
+    std::lock_guard<std::mutex> lock(g_comm_mu);
+    auto it = g_comms.find(key);
+    if (it != g_comms.end()) {
+        if (it->second.nranks != nranks || it->second.rank != rank || it->second.device != plan->dev.device) {
+            if (prev >= 0) cudaSetDevice(prev);
+            return fail(SEPCONV_E_INVALID, "NCCL id already used with a different rank, size or device");
+        }
+        ++it->second.refs;
+        plan->comm = it->second.comm;
+        if (prev >= 0) cudaSetDevice(prev);
+        return SEPCONV_OK;
+    }
     nccl_unique_id_t u;
     std::memcpy(u.internal, id, SEPCONV_NCCL_ID_BYTES);
     nccl_comm_t comm = nullptr;
     nccl_result_t r = a.CommInitRank(&comm, nranks, u, rank);
     if (prev >= 0) cudaSetDevice(prev);
     if (r != 0) return nccl_fail(r, "ncclCommInitRank");
+    SharedComm sc;
+    sc.comm = comm;
+    sc.nranks = nranks;
+    sc.rank = rank;
+    sc.refs = 1;
+    sc.device = plan->dev.device;
+    g_comms[key] = sc;
     plan->comm = comm;
     return SEPCONV_OK;
 }

@@ -275,3 +275,27 @@ def test_run_band_external_halo_equals_whole_image(G, K):
         torch.cuda.synchronize()
         got = torch.cat(parts, 0)
         assert torch.equal(got, want), v
+
+
+def test_run_band_nccl_single_rank_and_shared_comm():
+    """The NCCL path end to end on one GPU: the library dlopens the process's libnccl,
+    creates a unique id and a 1-rank communicator (no peers, so no send/recv is posted),
+    shares it between two plans, and run_band equals a plain run."""
+    H, W, K = 300, 700, 7
+    img = torch.from_numpy(synth.uniform_image(H, W, seed=41)).cuda()
+    k = synth.binomial_kernel(K)
+    uid = sc.nccl_unique_id()
+    assert len(uid) == sc.NCCL_ID_BYTES
+    p1, p2 = sc.Plan(H, W, K), sc.Plan(H, W, K)
+    p1.comm_init(uid, 1, 0)
+    p2.comm_init(uid, 1, 0)                               # same id: shared communicator
+    want = torch.empty((H - K + 1, W - K + 1), device="cuda")
+    p1.run(img, k, want, "separable")
+    for p in (p1, p2):
+        got = torch.empty_like(want)
+        band = img.clone()
+        p.run_band(band, k, got, "separable")
+        torch.cuda.synchronize()
+        assert torch.equal(got, want)
+    p1.close()
+    p2.close()
