@@ -465,6 +465,7 @@ sepconv_status_t sepconv_plan_ex(const sepconv_plan_desc_t *desc, sepconv_plan_t
         delete p;
         return cuda_fail(e, "cudaEventCreate");
     }
+    sepconv_seed_from_cache(p);
     *plan = p;
     return SEPCONV_OK;
 }

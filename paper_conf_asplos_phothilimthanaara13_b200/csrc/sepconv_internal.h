@@ -110,3 +110,4 @@ sepconv_status_t ensure_buf(sepconv_plan_t plan);
 }  // namespace sepconv
 
 void sepconv_comm_destroy_internal(sepconv_plan_t plan);   // sepconv_band.cpp
+void sepconv_seed_from_cache(sepconv_plan_t plan);         // sepconv_tune.cpp

@@ -115,7 +115,47 @@ void store_cache(const std::string &path, const std::string &key, const sepconv_
     std::rename(tmp.c_str(), path.c_str());
 }
 
+// The paper's selector picks a rule by input-size cutoffs (SELECT).  Here: a
+// plan of an untuned shape adopts the cached choice of the nearest tuned size (same GPU,
+// SM count, K and image count; sizes compared in log2 of the pixel count, within 2x).
+bool select_nearest(const std::string &path, sepconv_plan_t p, sepconv_choice_t best[3]) {
+    std::ifstream f(path);
+    if (!f) return false;
+    std::ostringstream pre;
+    pre << p->dev.name << "|" << p->dev.sms << "|";
+    const std::string want_pre = "\"key\":\"" + pre.str();
+    const double my = std::log2(static_cast<double>(p->h) * static_cast<double>(p->w));
+    double best_d = 1.0 + 1e-9;
+    bool found = false;
+    std::string line;
+    while (std::getline(f, line)) {
+        const size_t at = line.find(want_pre);
+        if (at == std::string::npos) continue;
+        long long n = 0, h = 0, w = 0;
+        int k = 0;
+        if (sscanf(line.c_str() + at + want_pre.size(), "%lldx%lldx%lld|k%d", &n, &h, &w, &k) != 4) continue;
+        if (k != p->k || n != p->n) continue;
+        const double d = std::fabs(std::log2(static_cast<double>(h) * static_cast<double>(w)) - my);
+        sepconv_choice_t b[3];
+        if (d < best_d && parse_choice(line, "2d", &b[0]) && parse_choice(line, "sep", &b[1]) &&
+            parse_choice(line, "auto", &b[2])) {
+            best_d = d;
+            std::memcpy(best, b, sizeof b);
+            found = true;
+        }
+    }
+    return found;
+}
+
 }  // namespace
+
+// Called by sepconv_plan_ex: an exact cache hit makes the plan tuned; otherwise the nearest
+// tuned size class (NEXT-2 of SURVEY 8(f)) seeds AUTO / 2D / SEPARABLE until sepconv_tune.
+void sepconv_seed_from_cache(sepconv_plan_t plan) {
+    const char *env = std::getenv("SEPCONV_TUNE_CACHE");
+    if (!env || !*env) return;
+    if (load_cache(env, cache_key(plan), plan->best) || select_nearest(env, plan, plan->best)) plan->tuned = true;
+}
 
 extern "C" {
 

@@ -299,3 +299,18 @@ def test_run_band_nccl_single_rank_and_shared_comm():
         assert torch.equal(got, want)
     p1.close()
     p2.close()
+
+
+def test_size_class_selector_seeds_untuned_plans(tmp_path, monkeypatch):
+    """NEXT-2: with $SEPCONV_TUNE_CACHE set, an untuned plan adopts the choice tuned for the
+    nearest image size (the paper's SELECT by input-size cutoffs)."""
+    cache = str(tmp_path / "tune.jsonl")
+    monkeypatch.setenv("SEPCONV_TUNE_CACHE", cache)
+    tuned = sc.Plan(1024, 1024, 9)
+    best = tuned.tune(reps=3, force=True)
+    near = sc.Plan(1100, 1000, 9)                          # 1.05x the pixels: same size class
+    assert near.get_choice("auto").key() == best.key()
+    far = sc.Plan(4096, 4096, 9)                           # 16x: not seeded
+    assert far.get_choice("auto").median_us == 0.0
+    img = synth.uniform_image(1100, 1000, seed=5)
+    check(img, synth.binomial_kernel(9), run_gpu(img, synth.binomial_kernel(9), variant="auto", plan=near)[0])
