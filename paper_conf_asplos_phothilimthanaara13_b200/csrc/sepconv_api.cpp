@@ -5,6 +5,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cmath>
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
@@ -181,13 +182,43 @@ static bool tma_ok(const float *base, long long ld, long long img) {
 // (64 x 4096^2: 4 strips x 64 images x 9 parts = 2304 items = 16 rounds of 144 CTAs).
 // Tiny problems (fewer rows than a part needs) fall back to the exactly balanced
 // contiguous split (parts = 0).
-static int schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K, int *parts) {
+//
+// When the strips do not divide the slots (16 CTA strips on 148 SMs at 16384^2: 144 CTAs,
+// 4 SMs idle -- 2.7% of the FP32 pipes the K >= 15 kernels are bound by), the window
+// schedule (parts = -q) keeps every slot busy: q windows of P rows one segment per CTA,
+// and the e = slots - q*S leftover CTAs share the short last window, m = ceil(S/e)
+// segments each; P solves P + o = m*(rows - q*P + o) (o = per-segment overhead in rows).
+// $SEPCONV_SCHED = "nowin" disables it, "win" forces it where eligible (tests, A/B runs).
+struct Sched {
+    int grid, parts, win_rows, extra;
+};
+
+static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K) {
     const long long slots = static_cast<long long>(di.sms) * occ;
     const long long strips = static_cast<long long>(nimg) * nstrips;
     const long long min_rows = std::max(8, 4 * (K - 1));
     const long long max_parts = std::max<long long>(1, rows / min_rows);
+    const double o = (K - 1) + 16.0;                           // warm-up + pipeline fill, rows
     double best = -1.0;
     long long best_p = 0, best_g = 0;
+    Sched win{0, 0, 0, 0};
+    double win_score = -1.0;
+    const char *mode = std::getenv("SEPCONV_SCHED");          // read per launch: tests flip it
+    const bool no_win = mode && std::strcmp(mode, "nowin") == 0;
+    const bool force_win = mode && std::strcmp(mode, "win") == 0;
+    if (!no_win && strips < slots && slots % strips != 0) {
+        const long long q = slots / strips, e = slots - q * strips;
+        const long long m = (strips + e - 1) / e;
+        long long P = static_cast<long long>(std::ceil((m * static_cast<double>(rows) + (m - 1) * o) / (m * q + 1)));
+        P = std::min<long long>(P, rows / q);
+        const long long L = rows - q * P;
+        if (P >= min_rows) {
+            const double makespan = std::max(P + o, L > 0 ? m * (L + o) : 0.0);
+            win_score = static_cast<double>(rows) * strips / (static_cast<double>(slots) * makespan);
+            win = Sched{static_cast<int>(q * strips + (L > 0 ? e : 0)), static_cast<int>(-q), static_cast<int>(P),
+                        static_cast<int>(L > 0 ? e : 0)};
+        }
+    }
     for (long long p = 1; p <= std::min<long long>(max_parts, 4096); ++p) {
         const long long items = strips * p;
         // grids to try: every slot, and the largest multiple of the strip count that fits
@@ -214,12 +245,10 @@ static int schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int ro
     const double contig_rows = static_cast<double>(total) / g_contig;
     const double contig_score = 0.92 * (contig_rows / (contig_rows + 2.0 * (K - 1 + 16))) *
                                 (static_cast<double>(g_contig) / slots);
-    if (best_p > 0 && best >= contig_score) {
-        *parts = static_cast<int>(best_p);
-        return static_cast<int>(best_g);
-    }
-    *parts = 0;
-    return static_cast<int>(std::max<long long>(g_contig, 1));
+    // the same model for the strided schedule: rounds x (segment rows + o)
+    if (win_score > 0 && (force_win || (win_score > best && win_score > contig_score))) return win;
+    if (best_p > 0 && best >= contig_score) return Sched{static_cast<int>(best_g), static_cast<int>(best_p), 0, 0};
+    return Sched{static_cast<int>(std::max<long long>(g_contig, 1)), 0, 0, 0};
 }
 
 // One streaming pass (ROWS, COLS or SEP) over geometry g.
@@ -270,8 +299,11 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
         if (s != SEPCONV_OK) return s;
     }
     if (p.total <= 0) return SEPCONV_OK;
-    const int grid = schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K, &p.parts);
-    cudaError_t e = stream_launch(op, map, K, smode, p, grid, st);
+    const Sched sc = schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K);
+    p.parts = sc.parts;
+    p.win_rows = sc.win_rows;
+    p.extra = sc.extra;
+    cudaError_t e = stream_launch(op, map, K, smode, p, sc.grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
     return SEPCONV_OK;
@@ -314,8 +346,11 @@ static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const 
         if (s != SEPCONV_OK) return s;
     }
     if (p.total <= 0) return SEPCONV_OK;
-    const int grid = schedule(plan->dev, occ, g.nimg, p.nstrips, g.rows, K, &p.parts);
-    cudaError_t e = conv2d_launch(map, K, p, grid, st);
+    const Sched sc = schedule(plan->dev, occ, g.nimg, p.nstrips, g.rows, K);
+    p.parts = sc.parts;
+    p.win_rows = sc.win_rows;
+    p.extra = sc.extra;
+    cudaError_t e = conv2d_launch(map, K, p, sc.grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "conv2d kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
     return SEPCONV_OK;

@@ -265,17 +265,47 @@ __device__ __forceinline__ void load_window_global(float (&x)[(XW + 3) & ~3], co
 //     (TLB- and L2-friendly: halo columns of neighbouring strips are read at the same time).
 //   parts = 0: CTA b takes the contiguous range [b*total/grid, (b+1)*total/grid) of the
 //     (image, strip, row) space -- exactly balanced, used when items would not divide evenly.
+//   parts = -q: every slot busy when the S = nimg*nstrips strips do not divide the slots:
+//     CTAs b < q*S take one segment each, rows [j*P, (j+1)*P) of strip b % S with
+//     j = b / S (q full-width windows of P = win_rows rows, strip-fastest as above); the
+//     e = extra remaining CTAs split the last window, rows [q*P, rows), CTA x taking the
+//     strips x, x+e, ...  The host sizes P so both kinds finish together.
 struct SegmentIter {
     long long total, u, u_end, item, items;
-    int rows, nstrips, parts;
-    __device__ SegmentIter(long long total_, int rows_, int nstrips_, int parts_, int nimg)
-        : total(total_), rows(rows_), nstrips(nstrips_), parts(parts_) {
+    int rows, nstrips, parts, win_rows, extra;
+    __device__ SegmentIter(long long total_, int rows_, int nstrips_, int parts_, int nimg, int win_rows_ = 0,
+                           int extra_ = 0)
+        : total(total_), rows(rows_), nstrips(nstrips_), parts(parts_), win_rows(win_rows_), extra(extra_) {
         u = total * blockIdx.x / gridDim.x;
         u_end = total * (blockIdx.x + 1) / gridDim.x;
         item = blockIdx.x;
         items = static_cast<long long>(nimg) * nstrips * (parts > 0 ? parts : 1);
     }
     __device__ bool next(int &n, int &s, int &q0, int &nrows) {
+        if (parts < 0) {
+            const long long S = items;                         // nimg * nstrips
+            const long long nmain = static_cast<long long>(-parts) * S;
+            long long sidx;
+            if (item < nmain) {                                // main CTA: one segment
+                sidx = item % S;
+                q0 = static_cast<int>((item / S) * win_rows);
+                nrows = win_rows;
+                item = nmain + S * extra;                      // done (never < nmain again)
+            } else {
+                // extra CTA x = blockIdx.x - nmain: item walks x, x + e, ... (offset by nmain)
+                if (item >= nmain + S * extra) return false;
+                const long long x = item - nmain;              // x + t*e on the t-th call
+                if (x >= S) return false;
+                sidx = x;
+                q0 = -parts * win_rows;
+                nrows = rows - q0;
+                if (nrows <= 0) return false;
+                item += extra;
+            }
+            n = static_cast<int>(sidx / nstrips);
+            s = static_cast<int>(sidx - static_cast<long long>(n) * nstrips);
+            return true;
+        }
         if (parts > 0) {
             if (item >= items) return false;
             s = static_cast<int>(item % nstrips);
@@ -337,7 +367,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         __syncwarp();
     }
 
-    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg);
+    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg, p.win_rows, p.extra);
     uint32_t kc = 0;                                           // chunks consumed by this warp
 
     int n, s, q0, nrows;
@@ -522,7 +552,7 @@ __global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constan
         __syncwarp();
     }
 
-    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg);
+    SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg, p.win_rows, p.extra);
     uint32_t kc = 0;
 
     int n, s, q0, nrows;

@@ -37,9 +37,12 @@ struct alignas(64) StreamParams {
     int rows;                    // output rows per image in this launch
     int nimg;
     int nstrips;                 // CTA strips = ceil(out_cols / (warps*128))
-    int parts;                   // >0: row partitions per (image, strip), strided schedule; 0: contiguous
+    int parts;                   // >0: row partitions per (image, strip), strided schedule; 0: contiguous;
+                                 // <0: -q full-width windows + extra CTAs (SegmentIter)
     int store8;                  // 2: every output row 16-byte aligned, 1: 8-byte aligned, 0: neither
     long long total;             // nimg * nstrips * rows (work units)
+    int win_rows;                // parts < 0: rows of each of the q main windows
+    int extra;                   // parts < 0: CTAs sharing the last (short) window
     float k[kMaxK];
     float2 k2[kMaxK];            // {k_i, k_i}: the same weights as packed-FP32 operands
 };
@@ -53,6 +56,7 @@ struct alignas(64) Conv2DParams {
     int in_rows, in_cols, out_cols;
     int row_begin, rows, nimg, nstrips, parts, store8;
     long long total;
+    int win_rows, extra;         // as StreamParams
     float w[kMaxK * kMaxK];      // w[j*K + i] = fl(k_i * k_j)
 };
 

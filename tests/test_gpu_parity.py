@@ -314,3 +314,35 @@ def test_size_class_selector_seeds_untuned_plans(tmp_path, monkeypatch):
     assert far.get_choice("auto").median_us == 0.0
     img = synth.uniform_image(1100, 1000, seed=5)
     check(img, synth.binomial_kernel(9), run_gpu(img, synth.binomial_kernel(9), variant="auto", plan=near)[0])
+
+
+# ---- work schedules: the window schedule (every SM busy) equals the others bit for bit -----
+@pytest.mark.parametrize("choice", [CANDS[0], CANDS[2], CANDS[3], CANDS[5], CANDS[6], CANDS[8]],
+                         ids=[IDS[i] for i in (0, 2, 3, 5, 6, 8)])
+def test_window_schedule_bitwise_and_parity(choice, monkeypatch):
+    """SEPCONV_SCHED=win forces the window schedule (q full-width windows + CTAs sharing the
+    short last window) wherever it is eligible; the schedule changes no pixel's arithmetic
+    (R6), so the output equals the strided/contiguous schedules' bitwise, and it
+    matches the oracle.  5 strips of 1024 columns on 148 SMs: q = 29, e = 3, m = 2."""
+    h, w = 2600, 5000
+    img = synth.uniform_image(h, w, seed=77)
+    dev = torch.from_numpy(img).cuda()
+    for K in (3, 10, 17):
+        k = synth.random_kernel(K, seed=K, signed=True)
+        p = sc.Plan(h, w, K)
+        outs = {}
+        for mode in ("nowin", "win"):
+            monkeypatch.setenv("SEPCONV_SCHED", mode)
+            out = torch.full((h - K + 1, w - K + 1), float("nan"), device="cuda")
+            p.run_choice(dev, k, out, choice)
+            torch.cuda.synchronize()
+            outs[mode] = out
+        monkeypatch.delenv("SEPCONV_SCHED")
+        assert not torch.isnan(outs["win"]).any().item(), f"K={K}: a cell was not written"
+        assert torch.equal(outs["win"], outs["nowin"]), f"K={K}"
+        rows = sorted({0, 1, 87, 88, 1000, h - K - 40, h - K - 1, h - K})
+        got = outs["win"][rows].cpu().numpy()
+        for i, r in enumerate(rows):
+            o, s = oracle.convolve2d(np.ascontiguousarray(img[r:r + K]), k, with_absum=True)
+            assert rel_error(got[i:i + 1], o, s) <= TOL, (K, r)
+        p.close()
