@@ -14,7 +14,8 @@ ap.add_argument("--n", type=int, default=2)
 ap.add_argument("--size", type=int, default=16384)
 a = ap.parse_args()
 names = {"sep-fused-tma0": (1, 1, 1, 0), "sep-fused-tma1": (1, 1, 1, 1), "sep-fused-tma2": (1, 1, 1, 2),
-         "sep-fused-tma3": (1, 1, 1, 3), "sep-fused-tma1s8": (1, 1, 1, 1, 1),
+         "sep-fused-tma3": (1, 1, 1, 3), "sep-fused-tma0s8": (1, 1, 1, 0, 1), "sep-fused-tma1s8": (1, 1, 1, 1, 1),
+         "sep-fused-tma2s8": (1, 1, 1, 2, 1), "sep-fused-tma3s8": (1, 1, 1, 3, 1),
          "sep-fused-direct": (1, 0, 1), "2d-tma": (0, 1, 0), "2d-direct": (0, 0, 0),
          "sep-unfused-tma": (1, 1, 0), "sep-unfused-direct": (1, 0, 0)}
 names["sep-fused-tma"] = names["sep-fused-tma0"]
