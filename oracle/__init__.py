@@ -1,4 +1,4 @@
-"""CPU oracle for SeparableConvolution -- TEST INFRASTRUCTURE ONLY.
+"""CPU oracles for SeparableConvolution and Poisson2D SOR -- TEST INFRASTRUCTURE ONLY.
 
 Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py``'s
 ``cpu_baseline`` / ``--impl reference`` legs may import this package.  The
@@ -11,7 +11,11 @@ only compiles it with gcc and marshals numpy arrays through ctypes.  The one
 piece of Python logic here, :func:`band_rows`, is the row-band partition
 reading of DESIGN.md R18 written out independently of the product's C code.
 
-Parity status: every function is pinned by ``tests/test_oracle_pins.py``.
+``poisson.c`` is the Poisson2D red-black SOR oracle (readings
+DESIGN.md section 11), wrapped by the ``sor_*`` / ``rb_*`` functions below.
+
+Parity status: every function is pinned by ``tests/test_oracle_pins.py`` and
+``tests/test_poisson_oracle.py``.
 """
 from __future__ import annotations
 
@@ -24,17 +28,18 @@ import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle.c")
+_SRCS = [_SRC, os.path.join(_HERE, "poisson.c")]
 _LIB = os.path.join(_HERE, "liboracle.so")
 _lock = threading.Lock()
 _lib = None
 
 
 def build(force: bool = False) -> str:
-    """Compile oracle.c into liboracle.so with plain gcc (-O2, no fast-math)."""
-    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
+    """Compile oracle.c + poisson.c into liboracle.so with plain gcc (-O2, no fast-math)."""
+    if force or not os.path.exists(_LIB) or any(os.path.getmtime(_LIB) < os.path.getmtime(s) for s in _SRCS):
         tmp = _LIB + ".tmp.%d" % os.getpid()
         subprocess.check_call(["gcc", "-O2", "-std=c11", "-fPIC", "-shared", "-pthread",
-                               "-fno-fast-math", "-ffp-contract=off", "-o", tmp, _SRC, "-lm"])
+                               "-fno-fast-math", "-ffp-contract=off", "-o", tmp, *_SRCS, "-lm"])
         os.replace(tmp, _LIB)
     return _LIB
 
@@ -53,8 +58,15 @@ def _load():
             lib.oracle_convolve_columns.argtypes = [f64p, i64, i64, f32p, i32, f64p]
             lib.oracle_separable.argtypes = [f32p, i64, i64, i64, f32p, i32, f64p, f64p]
             lib.oracle_num_cpus.argtypes = []
+            lib.oracle_sor_rb.argtypes = [f32p, f32p, i64, i64, ctypes.c_double, i32, f64p]
+            lib.oracle_sor_rb_f32.argtypes = [f32p, f32p, i64, i64, ctypes.c_float, i32, f32p]
+            lib.oracle_rb_split.argtypes = [f32p, i64, i64, f32p, f32p]
+            lib.oracle_rb_merge.argtypes = [f32p, f32p, i64, i64, f32p]
+            lib.oracle_poisson_residual.argtypes = [f64p, f32p, i64, i64, f64p]
             for fn in (lib.oracle_convolve2d, lib.oracle_convolve_rows,
-                       lib.oracle_convolve_columns, lib.oracle_separable, lib.oracle_num_cpus):
+                       lib.oracle_convolve_columns, lib.oracle_separable, lib.oracle_num_cpus,
+                       lib.oracle_sor_rb, lib.oracle_sor_rb_f32, lib.oracle_rb_split,
+                       lib.oracle_rb_merge, lib.oracle_poisson_residual):
                 fn.restype = ctypes.c_int
             _lib = lib
     return _lib
@@ -160,3 +172,85 @@ def convolve2d_bands(image, kernel, nbands: int):
         if r1 > r0:
             parts.append(convolve2d(np.ascontiguousarray(img[r0:r1 + K - 1]), k))
     return np.concatenate(parts, axis=0)
+
+
+# ---- Poisson2D red-black SOR (poisson.c) ----------------
+def _grid(x, name):
+    x = np.asarray(x)
+    if x.dtype != np.float32 or x.ndim != 2:
+        raise TypeError("%s must be a 2-D float32 matrix" % name)
+    return np.ascontiguousarray(x)
+
+
+def sor_rb(x, b, omega: float, iters: int):
+    """Red-black SOR (readings P1-P4) in double from the initial guess / boundary x and the
+    right-hand side b (both [N][M] float32); returns the iterate [N][M] float64."""
+    x, b = _grid(x, "x"), _grid(b, "b")
+    if x.shape != b.shape:
+        raise ValueError("x and b differ in shape")
+    u = np.empty(x.shape, np.float64)
+    if _load().oracle_sor_rb(x, b, x.shape[0], x.shape[1], float(omega), int(iters), u) != 0:
+        raise ValueError("oracle_sor_rb rejected its arguments")
+    return u
+
+
+def sor_rb_f32(x, b, omega: float, iters: int):
+    """The same iteration in float32 with the fixed evaluation order of DESIGN.md P6."""
+    x, b = _grid(x, "x"), _grid(b, "b")
+    if x.shape != b.shape:
+        raise ValueError("x and b differ in shape")
+    u = np.empty(x.shape, np.float32)
+    if _load().oracle_sor_rb_f32(x, b, x.shape[0], x.shape[1], float(np.float32(omega)), int(iters), u) != 0:
+        raise ValueError("oracle_sor_rb_f32 rejected its arguments")
+    return u
+
+
+def rb_split(x):
+    """Reading P5: red[i][k] = x[i][2k + (i & 1)], black[i][k] = x[i][2k + 1 - (i & 1)];
+    both [N][ceil(M/2)] (cells past the row's end are left 0)."""
+    x = _grid(x, "x")
+    n, m = x.shape
+    red = np.zeros((n, (m + 1) // 2), np.float32)
+    black = np.zeros_like(red)
+    if _load().oracle_rb_split(x, n, m, red, black) != 0:
+        raise ValueError("oracle_rb_split rejected its arguments")
+    return red, black
+
+
+def rb_merge(red, black, m: int):
+    red, black = _grid(red, "red"), _grid(black, "black")
+    n = red.shape[0]
+    x = np.empty((n, m), np.float32)
+    if _load().oracle_rb_merge(red, black, n, m, x) != 0:
+        raise ValueError("oracle_rb_merge rejected its arguments")
+    return x
+
+
+def poisson_residual(u, b):
+    """r = b - A u on interior cells (reading P1), 0 on the boundary frame; double."""
+    u = np.ascontiguousarray(np.asarray(u, np.float64))
+    b = _grid(b, "b")
+    r = np.empty(u.shape, np.float64)
+    if _load().oracle_poisson_residual(u, b, u.shape[0], u.shape[1], r) != 0:
+        raise ValueError("oracle_poisson_residual rejected its arguments")
+    return r
+
+
+def sor_abs_scale(x, b, omega: float, iters: int):
+    """The absolute-value iteration A_{t+1} = |1-w| A_t + (w/4) (sum |neighbours| + |b|),
+    A_0 = |x| (frame fixed): a per-cell bound on the magnitudes every float32 evaluation of
+    P4 combines, used to scale the rounding-error bound (P7): the red-black sweep
+    order of oracle_sor_rb with the coefficients |1-w| and w/4 applied to magnitudes."""
+    a = np.abs(_grid(x, "x")).astype(np.float64)
+    bb = np.abs(_grid(b, "b")).astype(np.float64)
+    n, m = a.shape
+    c0, c1 = abs(1.0 - omega), omega / 4.0
+    ii, jj = np.meshgrid(np.arange(n), np.arange(m), indexing="ij")
+    interior = (ii > 0) & (ii < n - 1) & (jj > 0) & (jj < m - 1)
+    masks = [interior & ((ii + jj) % 2 == c) for c in (0, 1)]
+    for _ in range(int(iters)):
+        for mask in masks:
+            nb = np.zeros_like(a)
+            nb[1:-1, 1:-1] = a[:-2, 1:-1] + a[2:, 1:-1] + a[1:-1, :-2] + a[1:-1, 2:]
+            a = np.where(mask, c0 * a + c1 * (nb + bb), a)
+    return a

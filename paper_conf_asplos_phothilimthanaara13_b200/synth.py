@@ -91,3 +91,26 @@ def delta_kernel(K: int, m: int) -> np.ndarray:
 
 def box_kernel(K: int, normalized: bool = False) -> np.ndarray:
     return np.full(K, (1.0 / K) if normalized else 1.0, np.float32)
+
+
+# ---- Poisson2D SOR inputs (input recipe) ------------------------------
+def poisson_problem(n: int, m: int, seed: int, guess: str = "zero"):
+    """(x, b) for an [n][m] grid: x carries the Dirichlet boundary (uniform [0,1) on the outer
+    frame) and the initial guess of the interior (0, or uniform [0,1) with guess="uniform");
+    b = f / (max(n, m) - 1)^2 with f uniform [0,1): the right-hand side with the grid spacing
+    h = 1/(max(n,m)-1) folded in (reading P1), so the solution is O(1)."""
+    u = uniform_image(n, m, seed, n=0)
+    x = np.zeros((n, m), np.float32)
+    x[0, :], x[-1, :], x[:, 0], x[:, -1] = u[0, :], u[-1, :], u[:, 0], u[:, -1]
+    if guess == "uniform" and n > 2 and m > 2:
+        x[1:-1, 1:-1] = u[1:-1, 1:-1]
+    h2 = float(max(n, m) - 1) ** 2 if max(n, m) > 1 else 1.0
+    b = (uniform_image(n, m, seed, n=1) / np.float32(h2)).astype(np.float32)
+    return x, b
+
+
+def omega_opt(n: int, m: int) -> float:
+    """Young's optimal relaxation factor for the model problem on the larger side,
+    2 / (1 + sin(pi / (max(n, m) - 1))) -- the bench's default w (an input, not a result)."""
+    s = max(n, m) - 1
+    return 2.0 / (1.0 + math.sin(math.pi / s)) if s > 1 else 1.0
