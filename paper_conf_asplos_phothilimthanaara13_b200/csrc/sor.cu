@@ -1,0 +1,602 @@
+// sor.cu -- Poisson2D red-black SOR on sm_100a (include/sor.h; PAPER.md P:1294-1308,
+// SURVEY.md 8(f) NEXT-3).
+//
+// Layout (reading P5): the plan splits x and b into red / black buffers, [N][ldh] each,
+// red[i][k] = x[i][2k + (i & 1)], black[i][k] = x[i][2k + 1 - (i & 1)].  In split
+// coordinates a cell (i, k) of colour c sits at grid column j = 2k + s, s = (i + c) & 1,
+// and its four neighbours are all of the other colour:
+//     N = other[i-1][k], S = other[i+1][k], W = other[i][k+s-1], E = other[i][k+s].
+//
+// Arithmetic (reading P6), identical in every kernel, bitwise equal to the fixed-order
+// float32 oracle:  t = (((N + S) + W) + E) + b;  u' = fma(w/4, t, (1-w) * u).
+//
+// Kernels:
+//   rb_split_kernel / rb_merge_kernel   P5 and its inverse (HBM-bound copies)
+//   sor_half_kernel<COLOR>              one half-sweep in place (SOR_HALF: 2 launches
+//                                       per iteration, 16 B of HBM traffic per cell)
+//   sor_wave_kernel<T>                  T iterations in one pass (SOR_WAVE): each warp
+//       owns a strip of 4*(32-2*HL) split columns (HL halo lanes per side, HL =
+//       ceil(2T/4): the dependency cone widens by one split column per half-sweep) and
+//       walks down its rows.  At step r it loads row r (level 0) and computes
+//       red_t(r-2t+1), black_t(r-2t) for t = 1..T from 3-row register windows of the
+//       previous level, so u and b are read once and u written once per T iterations
+//       (12 B per cell per pass), out of place into the plan's second buffer pair.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstring>
+#include <new>
+
+#include "../../include/sor.h"
+#include "sepconv_internal.h"
+
+namespace sor {
+
+constexpr int kMaxDepth = 8;
+constexpr int kWaveWarps = 4;            // warps per CTA of the wave kernel
+constexpr int kThreads = 256;            // split / merge / half kernels
+
+struct SorParams {
+    const float *ur, *ub;                // iterate read by the pass (split buffers)
+    float *ur_out, *ub_out;              // iterate written (HALF: the same buffers)
+    const float *br, *bb;                // right-hand side, split
+    long long ldh;                       // split row pitch (floats, multiple of 4)
+    int n, m;                            // grid rows, columns
+    float w4, om1;                       // w/4 and 1-w, formed in float32 on the host (P6)
+    int nstrips, seg_rows;               // wave schedule: items = nstrips * nsegs
+    long long items;
+};
+
+// interior columns of split quad k0..k0+3 for s = 0 (j = 2k) and s = 1 (j = 2k+1): bit e set
+// when 1 <= j <= m-2 (reading P2: the frame is never written)
+__device__ __forceinline__ unsigned col_mask(int k0, int s, int m, long long ldh) {
+    unsigned msk = 0;
+#pragma unroll
+    for (int e = 0; e < 4; ++e) {
+        const int k = k0 + e;
+        const int j = 2 * k + s;
+        if (k >= 0 && k < ldh && j >= 1 && j <= m - 2) msk |= 1u << e;
+    }
+    return msk;
+}
+
+__device__ __forceinline__ float relax1(float n, float s, float w, float e, float b, float u, float w4, float om1) {
+    float t = __fadd_rn(n, s);
+    t = __fadd_rn(t, w);
+    t = __fadd_rn(t, e);
+    t = __fadd_rn(t, b);
+    return __fmaf_rn(w4, t, __fmul_rn(om1, u));
+}
+
+// One quad of cells: u (own colour), N/S/C the other colour's rows i-1, i+1, i at the same
+// k, left = other[i][k0-1], right = other[i][k0+4]; s = row/colour parity, msk = interior
+// bits.  Cells outside the interior keep u.
+__device__ __forceinline__ float4 relax4(const float4 &u, const float4 &N, const float4 &S, const float4 &C,
+                                         float left, float right, const float4 &b, int s, unsigned msk, float w4,
+                                         float om1) {
+    const float W0 = s ? C.x : left, W1 = s ? C.y : C.x, W2 = s ? C.z : C.y, W3 = s ? C.w : C.z;
+    const float E0 = s ? C.y : C.x, E1 = s ? C.z : C.y, E2 = s ? C.w : C.z, E3 = s ? right : C.w;
+    float4 o;
+    o.x = (msk & 1u) ? relax1(N.x, S.x, W0, E0, b.x, u.x, w4, om1) : u.x;
+    o.y = (msk & 2u) ? relax1(N.y, S.y, W1, E1, b.y, u.y, w4, om1) : u.y;
+    o.z = (msk & 4u) ? relax1(N.z, S.z, W2, E2, b.z, u.z, w4, om1) : u.z;
+    o.w = (msk & 8u) ? relax1(N.w, S.w, W3, E3, b.w, u.w, w4, om1) : u.w;
+    return o;
+}
+
+__device__ __forceinline__ float4 ld4(const float *p) { return *reinterpret_cast<const float4 *>(p); }
+__device__ __forceinline__ float4 ldg4(const float *p) { return __ldg(reinterpret_cast<const float4 *>(p)); }
+__device__ __forceinline__ void st4(float *p, const float4 &v) { *reinterpret_cast<float4 *>(p) = v; }
+
+// ---- P5: split and merge ------------------------------------------------------------------
+// one thread per (row i, split quad k0..k0+3): grid columns 2k0 .. 2k0+7 of row i
+__global__ void rb_split_kernel(const float *__restrict__ x, long long ldx, int n, int m, float *__restrict__ red,
+                                float *__restrict__ black, long long ldh) {
+    const long long nq = ldh / 4;
+    for (long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; idx < n * nq;
+         idx += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int i = static_cast<int>(idx / nq);
+        const int k0 = static_cast<int>(idx - static_cast<long long>(i) * nq) * 4;
+        const float *row = x + i * ldx;
+        float v[8];
+#pragma unroll
+        for (int e = 0; e < 8; ++e) {
+            const int j = 2 * k0 + e;
+            v[e] = j < m ? row[j] : 0.f;
+        }
+        // row parity: red holds the even columns of even rows and the odd columns of odd rows
+        const int p = i & 1;
+        st4(red + i * ldh + k0, make_float4(v[p], v[2 + p], v[4 + p], v[6 + p]));
+        st4(black + i * ldh + k0, make_float4(v[1 - p], v[3 - p], v[5 - p], v[7 - p]));
+    }
+}
+
+__global__ void rb_merge_kernel(const float *__restrict__ red, const float *__restrict__ black, long long ldh, int n,
+                                int m, float *__restrict__ x, long long ldx) {
+    const long long nq = ldh / 4;
+    for (long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; idx < n * nq;
+         idx += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int i = static_cast<int>(idx / nq);
+        const int k0 = static_cast<int>(idx - static_cast<long long>(i) * nq) * 4;
+        const float4 r = ld4(red + i * ldh + k0), b = ld4(black + i * ldh + k0);
+        const int p = i & 1;
+        const float ev[4] = {p ? b.x : r.x, p ? b.y : r.y, p ? b.z : r.z, p ? b.w : r.w};   // even columns
+        const float od[4] = {p ? r.x : b.x, p ? r.y : b.y, p ? r.z : b.z, p ? r.w : b.w};   // odd columns
+        float *row = x + i * ldx;
+#pragma unroll
+        for (int e = 0; e < 4; ++e) {
+            const int j = 2 * (k0 + e);
+            if (j < m) row[j] = ev[e];
+            if (j + 1 < m) row[j + 1] = od[e];
+        }
+    }
+}
+
+// ---- SOR_HALF: one colour, in place -------------------------------------------------------
+template <int COLOR>
+__global__ void __launch_bounds__(kThreads) sor_half_kernel(const SorParams p) {
+    const long long nq = p.ldh / 4;
+    const long long rows = p.n - 2;
+    float *self = COLOR == 0 ? p.ur_out : p.ub_out;
+    const float *__restrict__ other = COLOR == 0 ? p.ub : p.ur;
+    const float *__restrict__ bs = COLOR == 0 ? p.br : p.bb;
+    for (long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; idx < rows * nq;
+         idx += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int i = 1 + static_cast<int>(idx / nq);
+        const int k0 = static_cast<int>(idx - static_cast<long long>(i - 1) * nq) * 4;
+        const int s = (i + COLOR) & 1;
+        const long long o = i * p.ldh + k0;
+        const float4 u = ld4(self + o);
+        const float4 b = ldg4(bs + o);
+        const float4 N = ldg4(other + o - p.ldh), S = ldg4(other + o + p.ldh), C = ldg4(other + o);
+        const float left = (s == 0 && k0 > 0) ? __ldg(other + o - 1) : 0.f;
+        const float right = (s == 1 && k0 + 4 < p.ldh) ? __ldg(other + o + 4) : 0.f;
+        st4(self + o, relax4(u, N, S, C, left, right, b, s, col_mask(k0, s, p.m, p.ldh), p.w4, p.om1));
+    }
+}
+
+// ---- SOR_WAVE: T iterations per pass ------------------------------------------------------
+template <int T>
+struct Wave {
+    static constexpr int HL = (2 * T + 3) / 4;       // halo lanes per side
+    static constexpr int OUT_LANES = 32 - 2 * HL;
+    static constexpr int WOUT = 4 * OUT_LANES;       // split columns written per strip
+};
+
+template <int T>
+__global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorParams p) {
+    constexpr int HL = Wave<T>::HL;
+    constexpr int WOUT = Wave<T>::WOUT;
+    const int lane = threadIdx.x & 31;
+    const long long gw = (blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x) >> 5;
+    const long long nw = (static_cast<long long>(gridDim.x) * blockDim.x) >> 5;
+    const int n = p.n;
+
+    for (long long item = gw; item < p.items; item += nw) {
+        const int strip = static_cast<int>(item % p.nstrips);
+        const int seg = static_cast<int>(item / p.nstrips);
+        const int q0 = seg * p.seg_rows;
+        const int q1 = min(n, q0 + p.seg_rows);
+        const int k0 = strip * WOUT - 4 * HL + 4 * lane;                 // this lane's first split column
+        const int kl = min(max(k0, 0), static_cast<int>(p.ldh) - 4);     // clamped for loads
+        const bool writer = lane >= HL && lane < 32 - HL && k0 < p.ldh;
+        const unsigned m0 = col_mask(k0, 0, p.m, p.ldh), m1 = col_mask(k0, 1, p.m, p.ldh);
+        // the wavefront starts 2T rows above the segment (aligned down to the window period 3)
+        int r0 = max(0, q0 - 2 * T);
+        r0 -= r0 % 3;
+        const int r_end = q1 - 1 + 2 * T;                                 // last step (inclusive)
+
+        float4 R[T + 1][3], B[T + 1][3];                                  // level windows, slot = row % 3
+#pragma unroll
+        for (int t = 0; t <= T; ++t)
+#pragma unroll
+            for (int z = 0; z < 3; ++z) R[t][z] = B[t][z] = make_float4(0.f, 0.f, 0.f, 0.f);
+
+        for (int rb = r0; rb <= r_end; rb += 3) {
+#pragma unroll
+            for (int u = 0; u < 3; ++u) {
+                const int r = rb + u;                                     // r % 3 == u
+                if (r < n) {
+                    const long long o = static_cast<long long>(r) * p.ldh + kl;
+                    R[0][u] = ldg4(p.ur + o);
+                    B[0][u] = ldg4(p.ub + o);
+                }
+#pragma unroll
+                for (int t = 1; t <= T; ++t) {
+                    // red_t at row rho = r - 2t + 1 from black_{t-1}(rho-1..rho+1), red_{t-1}(rho)
+                    {
+                        const int rho = r - 2 * t + 1;
+                        const int sc = ((u - 2 * t + 1) % 3 + 3) % 3;       // slot of rho (compile-time)
+                        const int sm = (sc + 2) % 3, sp = (sc + 1) % 3;
+                        const float4 C = B[t - 1][sc];
+                        const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
+                        const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
+                        const bool row_in = rho >= 1 && rho <= n - 2;
+                        const int s = rho & 1;
+                        const unsigned msk = row_in ? (s ? m1 : m0) : 0u;
+                        const float4 b = row_in ? ldg4(p.br + static_cast<long long>(rho) * p.ldh + kl)
+                                                : make_float4(0.f, 0.f, 0.f, 0.f);
+                        R[t][sc] = relax4(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, left, right, b, s, msk,
+                                          p.w4, p.om1);
+                    }
+                    // black_t at row beta = r - 2t from red_t(beta-1..beta+1), black_{t-1}(beta)
+                    {
+                        const int beta = r - 2 * t;
+                        const int sc = ((u - 2 * t) % 3 + 3) % 3;
+                        const int sm = (sc + 2) % 3, sp = (sc + 1) % 3;
+                        const float4 C = R[t][sc];
+                        const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
+                        const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
+                        const bool row_in = beta >= 1 && beta <= n - 2;
+                        const int s = (beta + 1) & 1;
+                        const unsigned msk = row_in ? (s ? m1 : m0) : 0u;
+                        const float4 b = row_in ? ldg4(p.bb + static_cast<long long>(beta) * p.ldh + kl)
+                                                : make_float4(0.f, 0.f, 0.f, 0.f);
+                        B[t][sc] = relax4(B[t - 1][sc], R[t][sm], R[t][sp], C, left, right, b, s, msk, p.w4,
+                                          p.om1);
+                    }
+                }
+                // finished rows of this step: red_T(r - 2T + 1), black_T(r - 2T)
+                if (writer) {
+                    const int rr = r - 2 * T + 1, br = r - 2 * T;
+                    if (rr >= q0 && rr < q1) st4(p.ur_out + static_cast<long long>(rr) * p.ldh + k0,
+                                                 R[T][((u - 2 * T + 1) % 3 + 3) % 3]);
+                    if (br >= q0 && br < q1) st4(p.ub_out + static_cast<long long>(br) * p.ldh + k0,
+                                                 B[T][((u - 2 * T) % 3 + 3) % 3]);
+                }
+            }
+        }
+    }
+}
+
+template <int T>
+cudaError_t launch_wave(const SorParams &p, int grid, cudaStream_t st) {
+    sor_wave_kernel<T><<<grid, kWaveWarps * 32, 0, st>>>(p);
+    return cudaGetLastError();
+}
+
+using WaveLaunch = cudaError_t (*)(const SorParams &, int, cudaStream_t);
+static const WaveLaunch kWave[kMaxDepth + 1] = {nullptr,         launch_wave<1>, launch_wave<2>,
+                                                launch_wave<3>,  launch_wave<4>, launch_wave<5>,
+                                                launch_wave<6>,  launch_wave<7>, launch_wave<8>};
+static const int kWout[kMaxDepth + 1] = {0,           Wave<1>::WOUT, Wave<2>::WOUT, Wave<3>::WOUT, Wave<4>::WOUT,
+                                         Wave<5>::WOUT, Wave<6>::WOUT, Wave<7>::WOUT, Wave<8>::WOUT};
+
+}  // namespace sor
+
+using sepconv::cuda_fail;
+using sepconv::fail;
+
+struct sor_plan_s {
+    int device = -1;
+    int sms = 0;
+    int64_t n = 0, m = 0, ldh = 0;
+    float *buf = nullptr;            // one allocation: 6 buffers of n * ldh floats
+    float *u[2][2] = {};             // [pair][colour]
+    float *b[2] = {};
+    int cur = 0;                     // pair holding the current iterate
+    int variant = -1, depth = 0;     // tuned (variant < 0: untuned)
+    int forced_depth = 0;
+    int wave_occ[sor::kMaxDepth + 1] = {};
+};
+
+namespace {
+
+constexpr int kDefaultDepth = 4;
+
+sepconv_status_t check_plan(sor_plan_t plan) {
+    if (!plan) return fail(SEPCONV_E_INVALID, "sor plan is NULL");
+    return SEPCONV_OK;
+}
+
+int grid_for(long long work, int threads, int sms) {
+    const long long blocks = (work + threads - 1) / threads;
+    return static_cast<int>(std::max<long long>(1, std::min<long long>(blocks, static_cast<long long>(sms) * 8)));
+}
+
+bool aligned16(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 15u) == 0; }
+
+sor::SorParams base_params(sor_plan_t plan, float omega) {
+    sor::SorParams p;
+    std::memset(&p, 0, sizeof p);
+    p.br = plan->b[0];
+    p.bb = plan->b[1];
+    p.ldh = plan->ldh;
+    p.n = static_cast<int>(plan->n);
+    p.m = static_cast<int>(plan->m);
+    p.w4 = omega * 0.25f;                      // exact (power-of-two scaling)
+    p.om1 = 1.0f - omega;                      // rounded once in float32 (P6)
+    return p;
+}
+
+sepconv_status_t half_iterations(sor_plan_t plan, float omega, int iters, cudaStream_t st) {
+    if (plan->n < 3 || plan->m < 3) return SEPCONV_OK;         // no interior
+    sor::SorParams p = base_params(plan, omega);
+    p.ur = p.ur_out = plan->u[plan->cur][0];
+    p.ub = p.ub_out = plan->u[plan->cur][1];
+    const int grid = grid_for((plan->n - 2) * (plan->ldh / 4), sor::kThreads, plan->sms);
+    for (int it = 0; it < iters; ++it) {
+        sor::sor_half_kernel<0><<<grid, sor::kThreads, 0, st>>>(p);
+        sor::sor_half_kernel<1><<<grid, sor::kThreads, 0, st>>>(p);
+        cudaError_t e = cudaGetLastError();
+        if (e != cudaSuccess) return cuda_fail(e, "sor_half_kernel launch");
+        sepconv::g_launches.fetch_add(2, std::memory_order_relaxed);
+    }
+    return SEPCONV_OK;
+}
+
+sepconv_status_t wave_pass(sor_plan_t plan, float omega, int T, cudaStream_t st) {
+    sor::SorParams p = base_params(plan, omega);
+    const int src = plan->cur, dst = 1 - plan->cur;
+    p.ur = plan->u[src][0];
+    p.ub = plan->u[src][1];
+    p.ur_out = plan->u[dst][0];
+    p.ub_out = plan->u[dst][1];
+    int &occ = plan->wave_occ[T];
+    if (occ == 0) {
+        static const void *funcs[sor::kMaxDepth + 1] = {
+            nullptr,
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<1>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<2>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<3>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<4>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<5>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<6>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<7>),
+            reinterpret_cast<const void *>(sor::sor_wave_kernel<8>)};
+        cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, funcs[T], sor::kWaveWarps * 32, 0);
+        if (e != cudaSuccess) return cuda_fail(e, "sor wave occupancy");
+        occ = std::max(occ, 1);
+    }
+    // items = strips x row segments, about one per resident warp (each segment pays 4T
+    // warm-up/drain steps: keep segments >= 16T rows)
+    p.nstrips = static_cast<int>((plan->ldh + sor::kWout[T] - 1) / sor::kWout[T]);
+    const long long warps = static_cast<long long>(plan->sms) * occ * sor::kWaveWarps;
+    long long nsegs = std::max<long long>(1, warps / p.nstrips);
+    nsegs = std::min<long long>(nsegs, std::max<long long>(1, plan->n / (16 * T)));
+    p.seg_rows = static_cast<int>((plan->n + nsegs - 1) / nsegs);
+    nsegs = (plan->n + p.seg_rows - 1) / p.seg_rows;
+    p.items = nsegs * p.nstrips;
+    const long long blocks = (p.items + sor::kWaveWarps - 1) / sor::kWaveWarps;
+    const int grid = static_cast<int>(std::min<long long>(blocks, static_cast<long long>(plan->sms) * occ));
+    cudaError_t e = sor::kWave[T](p, grid, st);
+    if (e != cudaSuccess) return cuda_fail(e, "sor_wave_kernel launch");
+    sepconv::g_launches.fetch_add(1, std::memory_order_relaxed);
+    plan->cur = dst;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t wave_iterations(sor_plan_t plan, float omega, int iters, int depth, cudaStream_t st) {
+    if (plan->n < 3 || plan->m < 3) return SEPCONV_OK;
+    while (iters > 0) {
+        const int T = std::min(iters, depth);
+        sepconv_status_t s = wave_pass(plan, omega, T, st);
+        if (s != SEPCONV_OK) return s;
+        iters -= T;
+    }
+    return SEPCONV_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+sepconv_status_t sor_plan(int64_t n, int64_t m, sor_plan_t *out) {
+    if (!out) return fail(SEPCONV_E_INVALID, "plan output pointer is NULL");
+    *out = nullptr;
+    if (n < 1 || m < 1 || n > (1LL << 30) || m > (1LL << 30))
+        return fail(SEPCONV_E_INVALID, "grid %lld x %lld: need 1 <= N, M <= 2^30", (long long)n, (long long)m);
+    int dev = 0, count = 0;
+    cudaError_t e = cudaGetDeviceCount(&count);
+    if (e != cudaSuccess || count == 0) return fail(SEPCONV_E_UNSUPPORTED, "no CUDA device");
+    SC_CUDA(cudaGetDevice(&dev));
+    cudaDeviceProp prop;
+    SC_CUDA(cudaGetDeviceProperties(&prop, dev));
+    if (prop.major != 10) return fail(SEPCONV_E_UNSUPPORTED, "device is sm_%d%d; built for sm_100a", prop.major, prop.minor);
+    sor_plan_t p = new (std::nothrow) sor_plan_s;
+    if (!p) return fail(SEPCONV_E_NOMEM, "host allocation");
+    p->device = dev;
+    p->sms = prop.multiProcessorCount;
+    p->n = n;
+    p->m = m;
+    p->ldh = (((m + 1) / 2) + 3) & ~3LL;
+    const size_t one = static_cast<size_t>(n) * static_cast<size_t>(p->ldh);
+    e = cudaMalloc(&p->buf, 6 * one * sizeof(float));
+    if (e != cudaSuccess) {
+        delete p;
+        return cuda_fail(e, "sor_plan workspace");
+    }
+    p->u[0][0] = p->buf;
+    p->u[0][1] = p->buf + one;
+    p->u[1][0] = p->buf + 2 * one;
+    p->u[1][1] = p->buf + 3 * one;
+    p->b[0] = p->buf + 4 * one;
+    p->b[1] = p->buf + 5 * one;
+    e = cudaMemset(p->buf, 0, 6 * one * sizeof(float));
+    if (e != cudaSuccess) {
+        cudaFree(p->buf);
+        delete p;
+        return cuda_fail(e, "sor_plan memset");
+    }
+    *out = p;
+    return SEPCONV_OK;
+}
+
+void sor_destroy(sor_plan_t plan) {
+    if (!plan) return;
+    cudaDeviceSynchronize();
+    cudaFree(plan->buf);
+    delete plan;
+}
+
+static bool overlaps(const void *a, size_t abytes, const void *b, size_t bbytes) {
+    const uintptr_t x = reinterpret_cast<uintptr_t>(a), y = reinterpret_cast<uintptr_t>(b);
+    return x < y + bbytes && y < x + abytes;
+}
+
+sepconv_status_t sor_load(sor_plan_t plan, const float *x, int64_t ld_x, const float *b, int64_t ld_b,
+                          sepconv_stream_t stream) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (!x || !b) return fail(SEPCONV_E_INVALID, "x or b is NULL");
+    ld_x = ld_x ? ld_x : plan->m;
+    ld_b = ld_b ? ld_b : plan->m;
+    if (ld_x < plan->m || ld_b < plan->m) return fail(SEPCONV_E_INVALID, "row pitch smaller than M");
+    if ((reinterpret_cast<uintptr_t>(x) | reinterpret_cast<uintptr_t>(b)) & 3u)
+        return fail(SEPCONV_E_ALIGN, "x and b must be 4-byte aligned");
+    const size_t ws = 6 * static_cast<size_t>(plan->n * plan->ldh) * sizeof(float);
+    if (overlaps(x, static_cast<size_t>(plan->n * ld_x) * 4, plan->buf, ws) ||
+        overlaps(b, static_cast<size_t>(plan->n * ld_b) * 4, plan->buf, ws))
+        return fail(SEPCONV_E_ALIAS, "x or b overlaps the plan's workspace");
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    const int grid = grid_for(plan->n * (plan->ldh / 4), sor::kThreads, plan->sms);
+    plan->cur = 0;
+    sor::rb_split_kernel<<<grid, sor::kThreads, 0, st>>>(x, ld_x, (int)plan->n, (int)plan->m, plan->u[0][0],
+                                                         plan->u[0][1], plan->ldh);
+    sor::rb_split_kernel<<<grid, sor::kThreads, 0, st>>>(b, ld_b, (int)plan->n, (int)plan->m, plan->b[0], plan->b[1],
+                                                         plan->ldh);
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(e, "rb_split_kernel launch");
+    sepconv::g_launches.fetch_add(2, std::memory_order_relaxed);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_iterate(sor_plan_t plan, float omega, int iters, sor_variant_t variant,
+                             sepconv_stream_t stream) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (!(omega > 0.f && omega < 2.f)) return fail(SEPCONV_E_INVALID, "omega %g outside (0, 2)", (double)omega);
+    if (iters < 0) return fail(SEPCONV_E_INVALID, "iters %d < 0", iters);
+    if (variant < SOR_HALF || variant > SOR_AUTO) return fail(SEPCONV_E_INVALID, "unknown variant %d", (int)variant);
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    int v = variant, depth = plan->forced_depth;
+    if (v == SOR_AUTO) v = plan->variant >= 0 ? plan->variant : SOR_WAVE;
+    if (depth == 0) depth = plan->depth > 0 ? plan->depth : kDefaultDepth;
+    return v == SOR_HALF ? half_iterations(plan, omega, iters, st) : wave_iterations(plan, omega, iters, depth, st);
+}
+
+sepconv_status_t sor_store(sor_plan_t plan, float *u, int64_t ld_u, sepconv_stream_t stream) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (!u) return fail(SEPCONV_E_INVALID, "u is NULL");
+    ld_u = ld_u ? ld_u : plan->m;
+    if (ld_u < plan->m) return fail(SEPCONV_E_INVALID, "row pitch smaller than M");
+    if (reinterpret_cast<uintptr_t>(u) & 3u) return fail(SEPCONV_E_ALIGN, "u must be 4-byte aligned");
+    const size_t ws = 6 * static_cast<size_t>(plan->n * plan->ldh) * sizeof(float);
+    if (overlaps(u, static_cast<size_t>(plan->n * ld_u) * 4, plan->buf, ws))
+        return fail(SEPCONV_E_ALIAS, "u overlaps the plan's workspace");
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    const int grid = grid_for(plan->n * (plan->ldh / 4), sor::kThreads, plan->sms);
+    sor::rb_merge_kernel<<<grid, sor::kThreads, 0, st>>>(plan->u[plan->cur][0], plan->u[plan->cur][1], plan->ldh,
+                                                         (int)plan->n, (int)plan->m, u, ld_u);
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(e, "rb_merge_kernel launch");
+    sepconv::g_launches.fetch_add(1, std::memory_order_relaxed);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_solve(sor_plan_t plan, const float *x, const float *b, float *u, float omega, int iters,
+                           sor_variant_t variant, sepconv_stream_t stream) {
+    if (sepconv_status_t s = sor_load(plan, x, 0, b, 0, stream)) return s;
+    if (sepconv_status_t s = sor_iterate(plan, omega, iters, variant, stream)) return s;
+    return sor_store(plan, u, 0, stream);
+}
+
+sepconv_status_t sor_solve_host(sor_plan_t plan, const float *x, const float *b, float *u, float omega, int iters,
+                                sor_variant_t variant, sepconv_stream_t stream) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (!x || !b || !u) return fail(SEPCONV_E_INVALID, "x, b or u is NULL");
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    const size_t bytes = static_cast<size_t>(plan->n * plan->m) * sizeof(float);
+    // staging: the second iterate pair (2 * N * ldh >= N * M floats, contiguous) is free
+    // before the first iteration -- x goes there and is split into pair 0, then b goes
+    // there and is split into the b buffers (stream order serialises the reuse)
+    float *stage = plan->u[1][0];
+    if (static_cast<size_t>(2 * plan->n * plan->ldh) * sizeof(float) < bytes)
+        return fail(SEPCONV_E_INVALID, "internal: staging too small");
+    const int grid = grid_for(plan->n * (plan->ldh / 4), sor::kThreads, plan->sms);
+    plan->cur = 0;
+    SC_CUDA(cudaMemcpyAsync(stage, x, bytes, cudaMemcpyHostToDevice, st));
+    sor::rb_split_kernel<<<grid, sor::kThreads, 0, st>>>(stage, plan->m, (int)plan->n, (int)plan->m, plan->u[0][0],
+                                                         plan->u[0][1], plan->ldh);
+    SC_CUDA(cudaGetLastError());
+    SC_CUDA(cudaMemcpyAsync(stage, b, bytes, cudaMemcpyHostToDevice, st));
+    sor::rb_split_kernel<<<grid, sor::kThreads, 0, st>>>(stage, plan->m, (int)plan->n, (int)plan->m, plan->b[0],
+                                                         plan->b[1], plan->ldh);
+    SC_CUDA(cudaGetLastError());
+    sepconv::g_launches.fetch_add(2, std::memory_order_relaxed);
+    if (sepconv_status_t s = sor_iterate(plan, omega, iters, variant, stream)) return s;
+    // merge into whichever pair is not current, then copy out
+    float *du = plan->u[1 - plan->cur][0];
+    sor::rb_merge_kernel<<<grid, sor::kThreads, 0, st>>>(plan->u[plan->cur][0], plan->u[plan->cur][1], plan->ldh,
+                                                         (int)plan->n, (int)plan->m, du, plan->m);
+    SC_CUDA(cudaGetLastError());
+    sepconv::g_launches.fetch_add(1, std::memory_order_relaxed);
+    SC_CUDA(cudaMemcpyAsync(u, du, bytes, cudaMemcpyDeviceToHost, st));
+    SC_CUDA(cudaStreamSynchronize(st));
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_buffers(sor_plan_t plan, float **u_red, float **u_black, float **b_red, float **b_black,
+                             int64_t *ldh) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (u_red) *u_red = plan->u[plan->cur][0];
+    if (u_black) *u_black = plan->u[plan->cur][1];
+    if (b_red) *b_red = plan->b[0];
+    if (b_black) *b_black = plan->b[1];
+    if (ldh) *ldh = plan->ldh;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_set_depth(sor_plan_t plan, int depth) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (depth < 0 || depth > sor::kMaxDepth) return fail(SEPCONV_E_INVALID, "depth %d outside 0..%d", depth, sor::kMaxDepth);
+    plan->forced_depth = depth;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_tune(sor_plan_t plan, int iters_hint, int reps, int *variant_out, int *depth_out) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (iters_hint < 1) iters_hint = 24;
+    if (reps < 1) reps = 5;
+    // time on the plan's own buffers (their contents are replaced by the caller's next load)
+    cudaStream_t st = nullptr;
+    cudaEvent_t e0, e1;
+    SC_CUDA(cudaEventCreate(&e0));
+    SC_CUDA(cudaEventCreate(&e1));
+    const int depths[] = {0, 1, 2, 3, 4, 5, 6, 8};       // 0 = SOR_HALF
+    float best = 1e30f;
+    int best_v = SOR_WAVE, best_d = kDefaultDepth;
+    const float omega = 1.5f;
+    sepconv_status_t status = SEPCONV_OK;
+    for (int d : depths) {
+        float times[64];
+        const int R = std::min(reps, 64);
+        for (int r = -1; r < R && status == SEPCONV_OK; ++r) {
+            cudaEventRecord(e0, st);
+            status = d == 0 ? half_iterations(plan, omega, iters_hint, st)
+                            : wave_iterations(plan, omega, iters_hint, d, st);
+            cudaEventRecord(e1, st);
+            if (cudaEventSynchronize(e1) != cudaSuccess) status = cuda_fail(cudaGetLastError(), "sor_tune");
+            float ms = 0.f;
+            cudaEventElapsedTime(&ms, e0, e1);
+            if (r >= 0) times[r] = ms;
+        }
+        if (status != SEPCONV_OK) break;
+        std::sort(times, times + R);
+        const float med = times[R / 2];
+        if (med < best * 0.99f) {
+            best = med;
+            best_v = d == 0 ? SOR_HALF : SOR_WAVE;
+            best_d = d == 0 ? kDefaultDepth : d;
+        }
+    }
+    cudaEventDestroy(e0);
+    cudaEventDestroy(e1);
+    if (status != SEPCONV_OK) return status;
+    plan->variant = best_v;
+    plan->depth = best_d;
+    if (variant_out) *variant_out = best_v;
+    if (depth_out) *depth_out = best_d;
+    return SEPCONV_OK;
+}
+
+}  // extern "C"

@@ -8,6 +8,7 @@ import pytest
 
 import oracle
 from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+from paper_conf_asplos_phothilimthanaara13_b200 import sor
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
@@ -24,6 +25,27 @@ def test_library_exports_every_declared_symbol():
     for name in declared:
         assert hasattr(L, name), name
     assert sorted(sc.exported_symbols()) == declared
+
+
+def test_library_exports_every_sor_symbol():
+    hdr = open(os.path.join(ROOT, "include", "sor.h")).read()
+    declared = sorted(set(re.findall(r"\b(sor_[a-z_]+)\s*\(", hdr)))
+    L = sor.lib()
+    assert len(declared) == 10
+    for name in declared:
+        assert hasattr(L, name), name
+    assert sorted(sor.exported_symbols()) == declared
+
+
+def test_sor_plan_validation_and_no_device():
+    with pytest.raises(sc.SepconvError) as ei:
+        sor.SorPlan(0, 5)
+    assert ei.value.code == "E_INVALID"
+    torch = pytest.importorskip("torch")
+    if not torch.cuda.is_available():
+        with pytest.raises(sc.SepconvError) as ei:
+            sor.SorPlan(64, 64)
+        assert ei.value.code == "E_UNSUPPORTED"
 
 
 def test_status_strings_and_version():

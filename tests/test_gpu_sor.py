@@ -1,0 +1,172 @@
+"""GPU parity for Poisson2D red-black SOR (include/sor.h)
+through the C ABI, against the CPU oracle (oracle/poisson.c).
+
+Bar: the split, the merge and every iterate are BIT-EXACT against the fixed-order float32
+oracle (reading P6) for every variant and wavefront depth; the iterate is also within the
+running-error bound (P7) of the double-precision definition.  Runs only on a B200 (-m gpu)."""
+import numpy as np
+import pytest
+
+import oracle
+from paper_conf_asplos_phothilimthanaara13_b200 import sor, synth
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+EPS32 = 2.0 ** -24
+
+
+def _dev(a):
+    return torch.from_numpy(np.ascontiguousarray(a)).cuda()
+
+
+class _Raw:
+    """A raw device pointer viewed as a float32 [rows][cols] tensor (no copy)."""
+
+    def __init__(self, ptr, rows, cols):
+        self.__cuda_array_interface__ = {"data": (int(ptr), False), "shape": (rows, cols),
+                                         "typestr": "<f4", "version": 2}
+
+
+def _split_from_device(p, n, m):
+    (ur, ub, br, bb), ldh = p.buffers()
+    torch.cuda.synchronize()
+    return [torch.as_tensor(_Raw(ptr, n, ldh), device="cuda").cpu().numpy()[:, :(m + 1) // 2]
+            for ptr in (ur, ub, br, bb)]
+
+
+def gpu_solve(x, b, omega, iters, variant="wave", depth=0, plan=None):
+    n, m = x.shape
+    p = plan or sor.SorPlan(n, m)
+    if depth:
+        p.set_depth(depth)
+    u = torch.full((n, m), float("nan"), device="cuda")
+    p.solve(_dev(x), _dev(b), u, omega, iters, variant)
+    torch.cuda.synchronize()
+    got = u.cpu().numpy()
+    assert not np.any(np.isnan(got)), "a cell of u was not written"
+    return got
+
+
+SHAPES = [(5, 5), (3, 3), (9, 14), (67, 131), (300, 1100), (1500, 300), (257, 1031)]
+
+
+def test_split_and_merge_bitwise():
+    for n, m in [(1, 1), (3, 5), (8, 9), (67, 131), (300, 1100)]:
+        x, b = synth.poisson_problem(n, m, seed=n + m, guess="uniform")
+        p = sor.SorPlan(n, m)
+        p.load(_dev(x), _dev(b))
+        ur, ub, br, bb = _split_from_device(p, n, m)
+        want_ur, want_ub = oracle.rb_split(x)
+        want_br, want_bb = oracle.rb_split(b)
+        # cells past a row's count of its colour are padding: compare the real cells only
+        cnt_red = [(m + 1 - (i & 1)) // 2 for i in range(n)]
+        cnt_black = [m // 2 if (i & 1) == 0 else (m + 1) // 2 for i in range(n)]
+        for got, want, cnt in ((ur, want_ur, cnt_red), (ub, want_ub, cnt_black), (br, want_br, cnt_red),
+                               (bb, want_bb, cnt_black)):
+            for i in range(n):
+                assert np.array_equal(got[i, :cnt[i]], want[i, :cnt[i]]), i
+        assert np.array_equal(oracle.rb_merge(ur, ub, m), x)
+        assert np.array_equal(oracle.rb_merge(br, bb, m), b)
+        u = torch.full((n, m), float("nan"), device="cuda")
+        p.store(u)
+        torch.cuda.synchronize()
+        assert np.array_equal(u.cpu().numpy(), x)                 # merge(split(x)) == x
+
+
+@pytest.mark.parametrize("shape", SHAPES, ids=lambda s: "%dx%d" % s)
+@pytest.mark.parametrize("variant,depth", [("half", 0), ("wave", 1), ("wave", 2), ("wave", 3), ("wave", 4),
+                                           ("wave", 5), ("wave", 8)])
+def test_iterates_bitwise_vs_f32_oracle(shape, variant, depth):
+    n, m = shape
+    x, b = synth.poisson_problem(n, m, seed=7 * n + m, guess="uniform")
+    omega = synth.omega_opt(n, m)
+    for iters in (1, 7):
+        got = gpu_solve(x, b, omega, iters, variant, depth)
+        want = oracle.sor_rb_f32(x, b, omega, iters)
+        assert np.array_equal(got, want), f"iters={iters}: max diff {np.max(np.abs(got - want))}"
+
+
+@pytest.mark.parametrize("omega", [0.7, 1.0, 1.5, 1.97])
+def test_within_running_error_bound_of_double(omega):
+    n, m, iters = 131, 77, 9
+    x, b = synth.poisson_problem(n, m, seed=3, guess="uniform")
+    got = gpu_solve(x, b, omega, iters, "auto")
+    u64 = oracle.sor_rb(x, b, omega, iters)
+    bound = 8 * EPS32 * iters * oracle.sor_abs_scale(x, b, omega, iters)
+    assert np.all(np.abs(got - u64) <= bound + 1e-30)
+
+
+def test_worked_example_on_gpu():
+    x = np.zeros((5, 5), np.float32)
+    b = np.zeros((5, 5), np.float32)
+    b[2, 2] = 4.0
+    want = np.zeros((5, 5), np.float32)
+    want[2, 2] = 1.25
+    want[1, 2] = want[2, 1] = want[2, 3] = want[3, 2] = 0.375
+    want[1, 1] = want[1, 3] = want[3, 1] = want[3, 3] = 0.125
+    for variant in ("half", "wave"):
+        assert np.array_equal(gpu_solve(x, b, 1.0, 2, variant), want)
+
+
+def test_degenerate_grids():
+    for n, m in ((1, 1), (2, 5), (5, 2), (1, 9), (3, 3)):
+        x, b = synth.poisson_problem(n, m, seed=1, guess="uniform")
+        for variant in ("half", "wave"):
+            got = gpu_solve(x, b, 1.5, 3, variant)
+            assert np.array_equal(got, oracle.sor_rb_f32(x, b, 1.5, 3))
+
+
+def test_harmonic_fixed_point_large_grid_exact():
+    """A discrete-harmonic integer field with b = 0 is a fixed point; at w = 1 every update
+    is exact in float32, so it must come back bit for bit (any index error breaks it)."""
+    n, m = 1030, 2050
+    i, j = np.meshgrid(np.arange(n, dtype=np.float64), np.arange(m, dtype=np.float64), indexing="ij")
+    h = (7.0 + 3.0 * i - 2.0 * j + i * j).astype(np.float32)          # |4u| < 2^24: exact
+    zero = np.zeros((n, m), np.float32)
+    for variant, depth in (("half", 0), ("wave", 4)):
+        assert np.array_equal(gpu_solve(h, zero, 1.0, 6, variant, depth), h)
+
+
+def test_solve_host_and_tune():
+    n, m = 300, 1100
+    x, b = synth.poisson_problem(n, m, seed=11, guess="uniform")
+    omega = synth.omega_opt(n, m)
+    p = sor.SorPlan(n, m)
+    v, d = p.tune(iters_hint=8, reps=3)
+    assert v in (sor.SOR_HALF, sor.SOR_WAVE) and 1 <= d <= sor.MAX_DEPTH
+    u = np.full((n, m), np.nan, np.float32)
+    p.solve_host(x, b, u, omega, 9, "auto")
+    assert np.array_equal(u, oracle.sor_rb_f32(x, b, omega, 9))
+
+
+def test_errors():
+    p = sor.SorPlan(16, 16)
+    x = torch.zeros((16, 16), device="cuda")
+    for omega, iters in ((0.0, 1), (2.0, 1), (1.5, -1)):
+        with pytest.raises(sor.SepconvError) as ei:
+            p.solve(x, x, torch.zeros_like(x), omega, iters)
+        assert ei.value.code == "E_INVALID"
+    with pytest.raises(sor.SepconvError) as ei:
+        p.set_depth(9)
+    assert ei.value.code == "E_INVALID"
+
+
+def test_sampled_blocks_at_bench_size():
+    """16384^2 (the bench's large grid) after 8 iterations: cells farther than 2T = 16 from
+    a crop's border depend only on the crop, so the oracle run on an even-offset crop (colour
+    parity preserved) gives them exactly (bitwise, float32 order P6)."""
+    n = m = 16384
+    iters = 8
+    x, b = synth.poisson_problem(n, m, seed=synth.BENCH_SEED_BASE + 40, guess="uniform")
+    got = gpu_solve(x, b, synth.omega_opt(n, m), iters, "auto")
+    margin = 2 * iters
+    for (i0, j0) in ((0, 0), (8190, 4096), (n - 160, m - 200), (0, m - 200), (5000, 0)):
+        h, w = 160, 200
+        cx = np.ascontiguousarray(x[i0:i0 + h, j0:j0 + w])
+        cb = np.ascontiguousarray(b[i0:i0 + h, j0:j0 + w])
+        want = oracle.sor_rb_f32(cx, cb, synth.omega_opt(n, m), iters)
+        top = 0 if i0 == 0 else margin
+        left = 0 if j0 == 0 else margin
+        bottom = h if i0 + h == n else h - margin
+        right = w if j0 + w == m else w - margin
+        assert np.array_equal(got[i0 + top:i0 + bottom, j0 + left:j0 + right], want[top:bottom, left:right]), (i0, j0)
