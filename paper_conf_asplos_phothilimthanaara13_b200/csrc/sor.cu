@@ -17,10 +17,12 @@
 //   sor_wave_kernel<T>                  T iterations in one pass (SOR_WAVE): each warp
 //       owns a strip of 4*(32-2*HL) split columns (HL halo lanes per side, HL =
 //       ceil(2T/4): the dependency cone widens by one split column per half-sweep) and
-//       walks down its rows.  At step r it loads row r (level 0) and computes
-//       red_t(r-2t+1), black_t(r-2t) for t = 1..T from 3-row register windows of the
-//       previous level, so u and b are read once and u written once per T iterations
-//       (12 B per cell per pass), out of place into the plan's second buffer pair.
+//       walks down its rows.  Rows arrive in a per-warp shared-memory ring by 1-D bulk
+//       copies (cp.async.bulk + mbarrier) PF rows ahead.  At step r the warp takes row
+//       r (level 0) and computes red_t(r-2t+1), black_t(r-2t) for t = 1..T from 3-row
+//       register windows of the previous level, so u and b are read once and u written
+//       once per T iterations (12 B per cell per pass), out of place into the plan's
+//       second buffer pair.
 #include <cuda_runtime.h>
 
 #include <algorithm>
@@ -66,7 +68,9 @@ __device__ __forceinline__ float relax1(float n, float s, float w, float e, floa
     t = __fadd_rn(t, w);
     t = __fadd_rn(t, e);
     t = __fadd_rn(t, b);
-    return __fmaf_rn(w4, t, __fmul_rn(om1, u));
+    // operands ordered so the uniform w/4 and 1-w sit in the constant-operand slot
+    // (FMUL/FFMA R, R, c[]); multiplication commutes exactly, so P6 is unchanged
+    return __fmaf_rn(t, w4, __fmul_rn(u, om1));
 }
 
 // One quad of cells: u (own colour), N/S/C the other colour's rows i-1, i+1, i at the same
@@ -88,6 +92,14 @@ __device__ __forceinline__ float4 relax4(const float4 &u, const float4 &N, const
 __device__ __forceinline__ float4 ld4(const float *p) { return *reinterpret_cast<const float4 *>(p); }
 __device__ __forceinline__ float4 ldg4(const float *p) { return __ldg(reinterpret_cast<const float4 *>(p)); }
 __device__ __forceinline__ void st4(float *p, const float4 &v) { *reinterpret_cast<float4 *>(p) = v; }
+// predicated 16-byte store: a branch-free body keeps ptxas from unswitching the hot loop
+__device__ __forceinline__ void st4_if(float *p, const float4 &v, bool ok) {
+    asm volatile(
+        "{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %5, 0;\n\t"
+        "@q st.global.v4.f32 [%0], {%1, %2, %3, %4};\n\t}" ::"l"(p),
+        "f"(v.x), "f"(v.y), "f"(v.z), "f"(v.w), "r"(static_cast<unsigned>(ok))
+        : "memory");
+}
 
 // ---- P5: split and merge ------------------------------------------------------------------
 // one thread per (row i, split quad k0..k0+3): grid columns 2k0 .. 2k0+7 of row i
@@ -162,97 +174,210 @@ struct Wave {
     static constexpr int HL = (2 * T + 3) / 4;       // halo lanes per side
     static constexpr int OUT_LANES = 32 - 2 * HL;
     static constexpr int WOUT = 4 * OUT_LANES;       // split columns written per strip
+    static constexpr int PF = 6;                     // rows prefetched ahead of the wavefront
+    static constexpr int RDU = 8;                    // u ring rows (>= PF + 1), one mbarrier each
+    // b ring rows: row r - 2T (black_T at step r) must survive until row r + PF lands
+    static constexpr int RDB = (2 * T + PF + 1 <= 16) ? 16 : 32;
+    static constexpr int WARP_FLOATS = 128 * (2 * RDU + 2 * RDB);
+    static constexpr size_t SMEM = static_cast<size_t>(kWaveWarps) * (WARP_FLOATS * 4 + RDU * 8);
+    static_assert(2 * T + PF + 1 <= RDB, "b ring too shallow");
 };
 
+__device__ __forceinline__ uint32_t smem_addr(const void *p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+__device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t bytes, uint64_t *bar) {
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                     smem_addr(dst)),
+                 "l"(src), "r"(bytes), "r"(smem_addr(bar))
+                 : "memory");
+}
+
+__device__ __forceinline__ void bar_expect(uint64_t *bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_addr(bar)), "r"(bytes) : "memory");
+}
+
+__device__ __forceinline__ void bar_wait(uint64_t *bar, uint32_t parity) {
+    uint32_t done, spins = 0;
+    do {
+        if (++spins == (1u << 26)) __trap();          // a lost transaction: fail loudly, never hang
+        asm volatile(
+            "{\n\t.reg .pred q;\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 q, [%1], %2;\n\t"
+            "selp.u32 %0, 1, 0, q;\n\t}"
+            : "=r"(done)
+            : "r"(smem_addr(bar)), "r"(parity)
+            : "memory");
+    } while (!done);
+}
+
+// relax4 with the parity a compile-time constant (the 6-step unroll fixes it)
+template <int S>
+__device__ __forceinline__ float4 relax4s(const float4 &u, const float4 &N, const float4 &Sv, const float4 &C,
+                                          float left, float right, const float4 &b, unsigned msk, float w4,
+                                          float om1) {
+    float4 o;
+    if constexpr (S == 0) {
+        o.x = (msk & 1u) ? relax1(N.x, Sv.x, left, C.x, b.x, u.x, w4, om1) : u.x;
+        o.y = (msk & 2u) ? relax1(N.y, Sv.y, C.x, C.y, b.y, u.y, w4, om1) : u.y;
+        o.z = (msk & 4u) ? relax1(N.z, Sv.z, C.y, C.z, b.z, u.z, w4, om1) : u.z;
+        o.w = (msk & 8u) ? relax1(N.w, Sv.w, C.z, C.w, b.w, u.w, w4, om1) : u.w;
+    } else {
+        o.x = (msk & 1u) ? relax1(N.x, Sv.x, C.x, C.y, b.x, u.x, w4, om1) : u.x;
+        o.y = (msk & 2u) ? relax1(N.y, Sv.y, C.y, C.z, b.y, u.y, w4, om1) : u.y;
+        o.z = (msk & 4u) ? relax1(N.z, Sv.z, C.z, C.w, b.z, u.z, w4, om1) : u.z;
+        o.w = (msk & 8u) ? relax1(N.w, Sv.w, C.w, right, b.w, u.w, w4, om1) : u.w;
+    }
+    return o;
+}
+
+// Rows reach shared memory through a per-warp ring filled by 1-D bulk copies (lane 0,
+// PF rows ahead, one mbarrier per u-ring slot covering the row's four copies: u red, u
+// black, b red, b black -- 512 B each); the b ring is deeper because the deepest level
+// still needs b of row r - 2T.  The step loop is unrolled 6 ways from a row that is a
+// multiple of 6, so the 3-row window slots (row % 3) and the row parities (which
+// neighbour column a cell needs, hence which single shuffle) are compile-time constants.
+// (Measured alternatives: waiting once per 6-row block lets steps
+// overlap but needs 36 KB of ring per warp -- 4 warps/SM -- and ran 20% slower.)
 template <int T>
 __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorParams p) {
-    constexpr int HL = Wave<T>::HL;
-    constexpr int WOUT = Wave<T>::WOUT;
-    const int lane = threadIdx.x & 31;
+    using WV = Wave<T>;
+    constexpr int HL = WV::HL, WOUT = WV::WOUT, PF = WV::PF, RDU = WV::RDU, RDB = WV::RDB;
+    extern __shared__ __align__(128) float wsmem[];
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    float *ring = wsmem + warp * WV::WARP_FLOATS;
+    float *ringU0 = ring, *ringU1 = ring + 128 * RDU;                     // u red, u black
+    float *ringB0 = ring + 256 * RDU, *ringB1 = ring + 256 * RDU + 128 * RDB;   // b red, b black
+    uint64_t *bars = reinterpret_cast<uint64_t *>(wsmem + kWaveWarps * WV::WARP_FLOATS) + warp * RDU;
+    if (lane == 0) {
+#pragma unroll
+        for (int i = 0; i < RDU; ++i)
+            asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(smem_addr(&bars[i])) : "memory");
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncwarp();
+
     const long long gw = (blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x) >> 5;
     const long long nw = (static_cast<long long>(gridDim.x) * blockDim.x) >> 5;
     const int n = p.n;
+    const long long ldh = p.ldh;
+    const unsigned nm2 = static_cast<unsigned>(n - 2);                  // row rho is interior iff rho-1 < n-2
+    uint32_t c = 0;                                                      // rows this warp has consumed
 
     for (long long item = gw; item < p.items; item += nw) {
         const int strip = static_cast<int>(item % p.nstrips);
         const int seg = static_cast<int>(item / p.nstrips);
         const int q0 = seg * p.seg_rows;
         const int q1 = min(n, q0 + p.seg_rows);
-        const int k0 = strip * WOUT - 4 * HL + 4 * lane;                 // this lane's first split column
-        const int kl = min(max(k0, 0), static_cast<int>(p.ldh) - 4);     // clamped for loads
-        const bool writer = lane >= HL && lane < 32 - HL && k0 < p.ldh;
-        const unsigned m0 = col_mask(k0, 0, p.m, p.ldh), m1 = col_mask(k0, 1, p.m, p.ldh);
-        // the wavefront starts 2T rows above the segment (aligned down to the window period 3)
+        const int kbase = strip * WOUT - 4 * HL;                          // lane 0's first split column
+        const int k0 = kbase + 4 * lane;
+        const bool writer = lane >= HL && lane < 32 - HL && k0 < ldh;
+        const unsigned m0 = col_mask(k0, 0, p.m, ldh), m1 = col_mask(k0, 1, p.m, ldh);
+        // the in-range part of the strip's 128 columns (bulk copies stay inside the rows)
+        const int g0 = max(kbase, 0), g1 = min(kbase + 128, static_cast<int>(ldh));
+        const uint32_t cbytes = static_cast<uint32_t>(g1 - g0) * 4u;
+        const int soff = g0 - kbase;
         int r0 = max(0, q0 - 2 * T);
-        r0 -= r0 % 3;
-        const int r_end = q1 - 1 + 2 * T;                                 // last step (inclusive)
+        r0 -= r0 % 6;
+        const int nsteps = ((q1 - 1 + 2 * T) - r0) / 6 * 6 + 6;           // whole 6-step blocks
+        const uint32_t c0 = c;
+        float *outR = p.ur_out + k0, *outB = p.ub_out + k0;
 
-        float4 R[T + 1][3], B[T + 1][3];                                  // level windows, slot = row % 3
+        auto issue = [&](int j) {                                        // step j = row r0 + j
+            const uint32_t cc = c0 + j;
+            uint64_t *bar = &bars[cc % RDU];
+            const int row = r0 + j;
+            if (row < n) {
+                const long long go = static_cast<long long>(row) * ldh + g0;
+                bar_expect(bar, 4 * cbytes);
+                bulk_g2s(ringU0 + (cc % RDU) * 128 + soff, p.ur + go, cbytes, bar);
+                bulk_g2s(ringU1 + (cc % RDU) * 128 + soff, p.ub + go, cbytes, bar);
+                bulk_g2s(ringB0 + (cc % RDB) * 128 + soff, p.br + go, cbytes, bar);
+                bulk_g2s(ringB1 + (cc % RDB) * 128 + soff, p.bb + go, cbytes, bar);
+            } else {
+                bar_expect(bar, 0);                                      // past the grid: complete the phase
+            }
+        };
+        __syncwarp();                                                    // every lane is past the last segment
+        if (lane == 0) {
+            asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+            for (int j = 0; j < min(PF, nsteps); ++j) issue(j);
+        }
+
+        float4 R[T + 1][3], B[T + 1][3];
 #pragma unroll
         for (int t = 0; t <= T; ++t)
 #pragma unroll
             for (int z = 0; z < 3; ++z) R[t][z] = B[t][z] = make_float4(0.f, 0.f, 0.f, 0.f);
 
-        for (int rb = r0; rb <= r_end; rb += 3) {
+#pragma unroll 1
+        for (int jb = 0; jb < nsteps; jb += 6) {
 #pragma unroll
-            for (int u = 0; u < 3; ++u) {
-                const int r = rb + u;                                     // r % 3 == u
-                if (r < n) {
-                    const long long o = static_cast<long long>(r) * p.ldh + kl;
-                    R[0][u] = ldg4(p.ur + o);
-                    B[0][u] = ldg4(p.ub + o);
+            for (int u = 0; u < 6; ++u) {
+                const int j = jb + u;
+                const int r = r0 + j;                                     // r % 6 == u
+                const uint32_t cc = c0 + j;
+                // refill: the slot row j+PF reuses was last read at step j-2 (u) / j-2 (b, row
+                // r+PF-RDB <= r-2T-1); all lanes are past step j-1 here
+                __syncwarp();
+                if (lane == 0 && j + PF < nsteps) {
+                    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+                    issue(j + PF);
                 }
+                bar_wait(&bars[cc % RDU], (cc / RDU) & 1);
+                __syncwarp();
+                R[0][u % 3] = *reinterpret_cast<const float4 *>(ringU0 + (cc % RDU) * 128 + 4 * lane);
+                B[0][u % 3] = *reinterpret_cast<const float4 *>(ringU1 + (cc % RDU) * 128 + 4 * lane);
 #pragma unroll
                 for (int t = 1; t <= T; ++t) {
-                    // red_t at row rho = r - 2t + 1 from black_{t-1}(rho-1..rho+1), red_{t-1}(rho)
-                    {
-                        const int rho = r - 2 * t + 1;
-                        const int sc = ((u - 2 * t + 1) % 3 + 3) % 3;       // slot of rho (compile-time)
-                        const int sm = (sc + 2) % 3, sp = (sc + 1) % 3;
+                    {   // red_t at rho = r - 2t + 1 (parity of u + 1)
+                        const int sc = ((u - 2 * t + 1) % 3 + 3) % 3, sm = (sc + 2) % 3, sp = (sc + 1) % 3;
                         const float4 C = B[t - 1][sc];
-                        const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
-                        const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
-                        const bool row_in = rho >= 1 && rho <= n - 2;
-                        const int s = rho & 1;
-                        const unsigned msk = row_in ? (s ? m1 : m0) : 0u;
-                        const float4 b = row_in ? ldg4(p.br + static_cast<long long>(rho) * p.ldh + kl)
-                                                : make_float4(0.f, 0.f, 0.f, 0.f);
-                        R[t][sc] = relax4(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, left, right, b, s, msk,
-                                          p.w4, p.om1);
+                        const bool row_in = static_cast<unsigned>(r - 2 * t) < nm2;   // rho - 1 < n - 2
+                        const float4 b = *reinterpret_cast<const float4 *>(
+                            ringB0 + ((cc - (2 * t - 1)) % RDB) * 128 + 4 * lane);
+                        if ((u + 1) % 2 == 0) {                             // rho even: red at even columns
+                            const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
+                            R[t][sc] = relax4s<0>(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, left, 0.f, b,
+                                                  row_in ? m0 : 0u, p.w4, p.om1);
+                        } else {
+                            const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
+                            R[t][sc] = relax4s<1>(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, 0.f, right, b,
+                                                  row_in ? m1 : 0u, p.w4, p.om1);
+                        }
                     }
-                    // black_t at row beta = r - 2t from red_t(beta-1..beta+1), black_{t-1}(beta)
-                    {
-                        const int beta = r - 2 * t;
-                        const int sc = ((u - 2 * t) % 3 + 3) % 3;
-                        const int sm = (sc + 2) % 3, sp = (sc + 1) % 3;
+                    {   // black_t at beta = r - 2t: black of row beta sits at column parity (beta+1)&1
+                        const int sc = ((u - 2 * t) % 3 + 3) % 3, sm = (sc + 2) % 3, sp = (sc + 1) % 3;
                         const float4 C = R[t][sc];
-                        const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
-                        const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
-                        const bool row_in = beta >= 1 && beta <= n - 2;
-                        const int s = (beta + 1) & 1;
-                        const unsigned msk = row_in ? (s ? m1 : m0) : 0u;
-                        const float4 b = row_in ? ldg4(p.bb + static_cast<long long>(beta) * p.ldh + kl)
-                                                : make_float4(0.f, 0.f, 0.f, 0.f);
-                        B[t][sc] = relax4(B[t - 1][sc], R[t][sm], R[t][sp], C, left, right, b, s, msk, p.w4,
-                                          p.om1);
+                        const bool row_in = static_cast<unsigned>(r - 2 * t - 1) < nm2;
+                        const float4 b = *reinterpret_cast<const float4 *>(
+                            ringB1 + ((cc - 2 * t) % RDB) * 128 + 4 * lane);
+                        if ((u + 1) % 2 == 0) {
+                            const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
+                            B[t][sc] = relax4s<0>(B[t - 1][sc], R[t][sm], R[t][sp], C, left, 0.f, b,
+                                                  row_in ? m0 : 0u, p.w4, p.om1);
+                        } else {
+                            const float right = __shfl_down_sync(0xffffffffu, C.x, 1);
+                            B[t][sc] = relax4s<1>(B[t - 1][sc], R[t][sm], R[t][sp], C, 0.f, right, b,
+                                                  row_in ? m1 : 0u, p.w4, p.om1);
+                        }
                     }
                 }
-                // finished rows of this step: red_T(r - 2T + 1), black_T(r - 2T)
-                if (writer) {
-                    const int rr = r - 2 * T + 1, br = r - 2 * T;
-                    if (rr >= q0 && rr < q1) st4(p.ur_out + static_cast<long long>(rr) * p.ldh + k0,
-                                                 R[T][((u - 2 * T + 1) % 3 + 3) % 3]);
-                    if (br >= q0 && br < q1) st4(p.ub_out + static_cast<long long>(br) * p.ldh + k0,
-                                                 B[T][((u - 2 * T) % 3 + 3) % 3]);
-                }
+                const int rr = r - 2 * T + 1, bt = r - 2 * T;
+                st4_if(outR + static_cast<long long>(rr) * ldh, R[T][((u - 2 * T + 1) % 3 + 3) % 3],
+                       writer && rr >= q0 && rr < q1);
+                st4_if(outB + static_cast<long long>(bt) * ldh, B[T][((u - 2 * T) % 3 + 3) % 3],
+                       writer && bt >= q0 && bt < q1);
             }
         }
+        c = c0 + nsteps;
     }
 }
 
 template <int T>
 cudaError_t launch_wave(const SorParams &p, int grid, cudaStream_t st) {
-    sor_wave_kernel<T><<<grid, kWaveWarps * 32, 0, st>>>(p);
+    sor_wave_kernel<T><<<grid, kWaveWarps * 32, Wave<T>::SMEM, st>>>(p);
     return cudaGetLastError();
 }
 
@@ -283,7 +408,7 @@ struct sor_plan_s {
 
 namespace {
 
-constexpr int kDefaultDepth = 4;
+constexpr int kDefaultDepth = 3;      // measured best at 16384^2 (profiles/r01_sor_perf.txt)
 
 sepconv_status_t check_plan(sor_plan_t plan) {
     if (!plan) return fail(SEPCONV_E_INVALID, "sor plan is NULL");
@@ -345,7 +470,14 @@ sepconv_status_t wave_pass(sor_plan_t plan, float omega, int T, cudaStream_t st)
             reinterpret_cast<const void *>(sor::sor_wave_kernel<6>),
             reinterpret_cast<const void *>(sor::sor_wave_kernel<7>),
             reinterpret_cast<const void *>(sor::sor_wave_kernel<8>)};
-        cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, funcs[T], sor::kWaveWarps * 32, 0);
+        static const size_t smem[sor::kMaxDepth + 1] = {0,
+                                                        sor::Wave<1>::SMEM, sor::Wave<2>::SMEM, sor::Wave<3>::SMEM,
+                                                        sor::Wave<4>::SMEM, sor::Wave<5>::SMEM, sor::Wave<6>::SMEM,
+                                                        sor::Wave<7>::SMEM, sor::Wave<8>::SMEM};
+        cudaError_t e = cudaFuncSetAttribute(funcs[T], cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                             static_cast<int>(smem[T]));
+        if (e != cudaSuccess) return cuda_fail(e, "sor wave smem attribute");
+        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, funcs[T], sor::kWaveWarps * 32, smem[T]);
         if (e != cudaSuccess) return cuda_fail(e, "sor wave occupancy");
         occ = std::max(occ, 1);
     }
