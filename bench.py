@@ -10,7 +10,8 @@ of the image per width (8 passes of the whole hot path), each with the tuned AUT
 variant.  At N > 1 (torchrun) the image is split into N row bands, one per GPU, and
 every pass exchanges the (K-1)-row halo with NCCL send/recv inside the C ABI
 (sepconv_run_band); scaling is strong (fixed image).  --workload batch is
-configs[4] (64 x 4096^2, K = 11, images sharded over ranks, no exchange).
+configs[4] (64 x 4096^2, K = 11, images sharded over ranks, no exchange).  --workload
+poisson is the NEXT-3 Poisson2D red-black SOR leg (bench_poisson.py).
 
 value = output pixels of the whole job per step / max-over-ranks device time
 (CUDA events, inputs resident in HBM; the 1.07 GB image is larger than the 126 MB
@@ -48,7 +49,7 @@ def parse_args():
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--workload", choices=["image", "batch"], default="image")
+    ap.add_argument("--workload", choices=["image", "batch", "poisson"], default="image")
     ap.add_argument("--widths", default="3,5,7,9,11,13,15,17")
     ap.add_argument("--size", type=int, default=16384, help="image side (image workload)")
     ap.add_argument("--variant", default="auto")
@@ -56,6 +57,7 @@ def parse_args():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle time for the cpu_baseline sample")
     ap.add_argument("--tune-reps", type=int, default=10)
+    ap.add_argument("--sor-iters", type=int, default=24, help="poisson workload: iterations per step")
     return ap.parse_args()
 
 
@@ -201,6 +203,9 @@ def run_reference(args):
 # --------------------------------------------------------------------------------------------
 def main():
     args = parse_args()
+    if args.workload == "poisson":
+        import bench_poisson
+        return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit)
     if args.impl == "reference":
         return run_reference(args)
 
