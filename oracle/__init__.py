@@ -12,10 +12,12 @@ piece of Python logic here, :func:`band_rows`, is the row-band partition
 reading of DESIGN.md R18 written out independently of the product's C code.
 
 ``poisson.c`` is the Poisson2D red-black SOR oracle (readings
-DESIGN.md section 11), wrapped by the ``sor_*`` / ``rb_*`` functions below.
+DESIGN.md section 11), wrapped by the ``sor_*`` / ``rb_*`` functions below;
+``blackscholes.c`` the Black-Scholes oracle,
+wrapped by :func:`black_scholes`.
 
 Parity status: every function is pinned by ``tests/test_oracle_pins.py`` and
-``tests/test_poisson_oracle.py``.
+``tests/test_poisson_oracle.py`` and ``tests/test_bs_oracle.py``.
 """
 from __future__ import annotations
 
@@ -28,14 +30,14 @@ import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle.c")
-_SRCS = [_SRC, os.path.join(_HERE, "poisson.c")]
+_SRCS = [_SRC, os.path.join(_HERE, "poisson.c"), os.path.join(_HERE, "blackscholes.c")]
 _LIB = os.path.join(_HERE, "liboracle.so")
 _lock = threading.Lock()
 _lib = None
 
 
 def build(force: bool = False) -> str:
-    """Compile oracle.c + poisson.c into liboracle.so with plain gcc (-O2, no fast-math)."""
+    """Compile oracle.c, poisson.c and blackscholes.c into liboracle.so (gcc -O2, no fast-math)."""
     if force or not os.path.exists(_LIB) or any(os.path.getmtime(_LIB) < os.path.getmtime(s) for s in _SRCS):
         tmp = _LIB + ".tmp.%d" % os.getpid()
         subprocess.check_call(["gcc", "-O2", "-std=c11", "-fPIC", "-shared", "-pthread",
@@ -63,10 +65,12 @@ def _load():
             lib.oracle_rb_split.argtypes = [f32p, i64, i64, f32p, f32p]
             lib.oracle_rb_merge.argtypes = [f32p, f32p, i64, i64, f32p]
             lib.oracle_poisson_residual.argtypes = [f64p, f32p, i64, i64, f64p]
+            lib.oracle_black_scholes.argtypes = [f32p, f32p, f32p, i64, ctypes.c_double, ctypes.c_double,
+                                                 f64p, f64p, ctypes.c_void_p]
             for fn in (lib.oracle_convolve2d, lib.oracle_convolve_rows,
                        lib.oracle_convolve_columns, lib.oracle_separable, lib.oracle_num_cpus,
                        lib.oracle_sor_rb, lib.oracle_sor_rb_f32, lib.oracle_rb_split,
-                       lib.oracle_rb_merge, lib.oracle_poisson_residual):
+                       lib.oracle_rb_merge, lib.oracle_poisson_residual, lib.oracle_black_scholes):
                 fn.restype = ctypes.c_int
             _lib = lib
     return _lib
@@ -254,3 +258,20 @@ def sor_abs_scale(x, b, omega: float, iters: int):
             nb[1:-1, 1:-1] = a[:-2, 1:-1] + a[2:, 1:-1] + a[1:-1, :-2] + a[1:-1, 2:]
             a = np.where(mask, c0 * a + c1 * (nb + bb), a)
     return a
+
+
+# ---- Black-Scholes (blackscholes.c) -----------------------
+def black_scholes(s, x, t, r: float, v: float, with_scale: bool = False):
+    """European call and put prices in double for float32 spot s, strike x, expiry t (years)
+    and scalar rate r, volatility v; optionally the float32 error scale of reading B4."""
+    s, x, t = (np.ascontiguousarray(np.asarray(a, np.float32).reshape(-1)) for a in (s, x, t))
+    if not (s.size == x.size == t.size):
+        raise ValueError("s, x, t differ in length")
+    call = np.empty(s.size, np.float64)
+    put = np.empty(s.size, np.float64)
+    scale = np.empty(s.size, np.float64) if with_scale else None
+    rc = _load().oracle_black_scholes(s, x, t, s.size, float(r), float(v), call, put,
+                                      scale.ctypes.data if with_scale else None)
+    if rc != 0:
+        raise ValueError("oracle_black_scholes rejected its arguments")
+    return (call, put, scale) if with_scale else (call, put)

@@ -114,3 +114,18 @@ def omega_opt(n: int, m: int) -> float:
     2 / (1 + sin(pi / (max(n, m) - 1))) -- the bench's default w (an input, not a result)."""
     s = max(n, m) - 1
     return 2.0 / (1.0 + math.sin(math.pi / s)) if s > 1 else 1.0
+
+
+# ---- Black-Scholes inputs (DESIGN.md section 12, input recipe) ------------------------------
+BS_RATE, BS_VOL = 0.02, 0.30
+
+
+def bs_options(n: int, seed: int):
+    """(spot, strike, years) float32 arrays of n options from the counter generator:
+    S uniform [5, 30), X uniform [1, 100), T uniform [0.25, 10) -- the ranges of the
+    classic GPU Black-Scholes benchmark; r = BS_RATE, v = BS_VOL are scalars."""
+    u = uniform_image(3, n, seed)
+    s = (np.float32(5.0) + np.float32(25.0) * u[0]).astype(np.float32)
+    x = (np.float32(1.0) + np.float32(99.0) * u[1]).astype(np.float32)
+    t = (np.float32(0.25) + np.float32(9.75) * u[2]).astype(np.float32)
+    return s, x, t

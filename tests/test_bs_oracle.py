@@ -1,0 +1,110 @@
+"""Pins for the Black-Scholes oracle (oracle/blackscholes.c, readings
+DESIGN.md section 12): a textbook worked example (tests/golden/bs_hull.txt), put-call parity,
+the zero-volatility / zero-time limits (intrinsic value of the forward), the deep in/out of
+the money limits, delta = N(d1) by central finite differences, monotonicity in S, X and v,
+and the float32 error-scale bound.  None re-types the formula.  CPU only."""
+import math
+import os
+
+import numpy as np
+import pytest
+
+import oracle
+from paper_conf_asplos_phothilimthanaara13_b200 import synth
+
+GOLDEN = os.path.join(os.path.dirname(__file__), "golden")
+
+
+def _golden():
+    d = {}
+    for line in open(os.path.join(GOLDEN, "bs_hull.txt")):
+        if line.strip() and not line.startswith("#"):
+            k, v = line.split()
+            d[k] = float(v)
+    return d
+
+
+def test_textbook_worked_example():
+    g = _golden()
+    c, p = oracle.black_scholes([g["S"]], [g["X"]], [g["T"]], g["r"], g["v"])
+    assert abs(c[0] - g["call"]) <= 0.005 and abs(p[0] - g["put"]) <= 0.005
+
+
+def test_put_call_parity():
+    s, x, t = synth.bs_options(4096, seed=5)
+    r, v = synth.BS_RATE, synth.BS_VOL
+    c, p = oracle.black_scholes(s, x, t, r, v)
+    lhs = c - p
+    rhs = s.astype(np.float64) - x.astype(np.float64) * np.exp(-r * t.astype(np.float64))
+    assert np.max(np.abs(lhs - rhs)) <= 1e-12 * np.max(np.abs(rhs) + 1)
+
+
+@pytest.mark.parametrize("r", [0.0, 0.05])
+def test_small_volatility_and_time_limits_are_intrinsic(r):
+    """v -> 0: the call tends to max(S - X e^{-rT}, 0) (no uncertainty left)."""
+    s = np.array([10, 20, 30, 50, 50.5], np.float32)
+    x = np.array([20, 20, 20, 50, 50], np.float32)
+    t = np.full(5, 1.0, np.float32)
+    c, p = oracle.black_scholes(s, x, t, r, 1e-6)
+    fwd = s.astype(np.float64) - x.astype(np.float64) * math.exp(-r)
+    # the gap closes like S v sqrt(T / 2 pi) at the money: <= 2e-5 here
+    assert np.allclose(c, np.maximum(fwd, 0), atol=1e-4, rtol=0)
+    assert np.allclose(p, np.maximum(-fwd, 0), atol=1e-4, rtol=0)
+    c2, _ = oracle.black_scholes(s, x, np.full(5, 1e-10, np.float32), r, 0.3)
+    assert np.allclose(c2, np.maximum(s.astype(np.float64) - x, 0), atol=1e-3)
+
+
+def test_deep_in_and_out_of_the_money():
+    c, p = oracle.black_scholes([1000.0, 1.0], [1.0, 1000.0], [1.0, 1.0], 0.03, 0.2)
+    assert c[0] == pytest.approx(1000.0 - math.exp(-0.03), rel=1e-12)
+    assert c[1] < 1e-100 and p[1] == pytest.approx(1000.0 * math.exp(-0.03) - 1.0, rel=1e-12)
+
+
+def test_delta_is_n_of_d1():
+    """dC/dS = N(d1): a central difference of the oracle against N(d1) evaluated with
+    math.erfc (pins d1, the CDF and the sign of every term)."""
+    S, X, T, r, v = 23.0, 25.0, 1.5, 0.04, 0.35
+    h = 1e-3
+    cu, _ = oracle.black_scholes([np.float32(S + h)], [X], [T], r, v)
+    cd, _ = oracle.black_scholes([np.float32(S - h)], [X], [T], r, v)
+    sp, sm = float(np.float32(S + h)), float(np.float32(S - h))
+    delta = (cu[0] - cd[0]) / (sp - sm)
+    d1 = (math.log(S / X) + (r + v * v / 2) * T) / (v * math.sqrt(T))
+    assert delta == pytest.approx(0.5 * math.erfc(-d1 / math.sqrt(2)), abs=1e-6)
+
+
+def test_monotone_in_spot_strike_and_volatility():
+    s = np.linspace(5, 30, 64, dtype=np.float32)
+    c, p = oracle.black_scholes(s, np.full(64, 17, np.float32), np.full(64, 2, np.float32), 0.02, 0.3)
+    assert np.all(np.diff(c) > 0) and np.all(np.diff(p) < 0)
+    x = np.linspace(1, 100, 64, dtype=np.float32)
+    c, p = oracle.black_scholes(np.full(64, 17, np.float32), x, np.full(64, 2, np.float32), 0.02, 0.3)
+    assert np.all(np.diff(c) < 0) and np.all(np.diff(p) > 0)
+    lo = oracle.black_scholes([17], [20], [2], 0.02, 0.2)[0][0]
+    hi = oracle.black_scholes([17], [20], [2], 0.02, 0.4)[0][0]
+    assert hi > lo                                               # vega > 0
+
+
+def test_error_scale_bounds_a_float32_evaluation():
+    """A float32 evaluation of the same formula (numpy, float32 throughout, erfc from
+    math in double then rounded) stays within 16 eps x the oracle's B4 error scale."""
+    s, x, t = synth.bs_options(2000, seed=9)
+    r, v = np.float32(synth.BS_RATE), np.float32(synth.BS_VOL)
+    c, p, scale = oracle.black_scholes(s, x, t, float(r), float(v), with_scale=True)
+    sq = np.sqrt(t)
+    d1 = (np.log(s / x) + (r + np.float32(0.5) * v * v) * t) / (v * sq)
+    d2 = d1 - v * sq
+    n = np.vectorize(lambda z: np.float32(0.5 * math.erfc(-float(z) / math.sqrt(2))), otypes=[np.float32])
+    disc = x * np.exp(-r * t)
+    c32 = s * n(d1) - disc * n(d2)
+    p32 = disc * n(-d2) - s * n(-d1)
+    eps = 2.0 ** -24
+    assert np.all(np.abs(c32 - c) <= 16 * eps * scale)
+    assert np.all(np.abs(p32 - p) <= 16 * eps * scale)
+
+
+def test_rejects_invalid_inputs():
+    with pytest.raises(ValueError):
+        oracle.black_scholes([1.0], [0.0], [1.0], 0.02, 0.3)
+    with pytest.raises(ValueError):
+        oracle.black_scholes([1.0], [1.0], [1.0], 0.02, 0.0)
