@@ -8,7 +8,7 @@ import pytest
 
 import oracle
 from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
-from paper_conf_asplos_phothilimthanaara13_b200 import sor
+from paper_conf_asplos_phothilimthanaara13_b200 import bs, sor
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
@@ -35,6 +35,23 @@ def test_library_exports_every_sor_symbol():
     for name in declared:
         assert hasattr(L, name), name
     assert sorted(sor.exported_symbols()) == declared
+
+
+def test_library_exports_every_bs_symbol():
+    hdr = open(os.path.join(ROOT, "include", "bs.h")).read()
+    declared = sorted(set(re.findall(r"\b(bs_[a-z_]+)\s*\(", hdr)))
+    L = bs.lib()
+    assert declared == sorted(bs.exported_symbols())
+    for name in declared:
+        assert hasattr(L, name), name
+
+
+def test_bs_validation_before_device():
+    import numpy as np
+    a = np.ones(8, np.float32)
+    with pytest.raises(sc.SepconvError) as ei:
+        bs.price(a.ctypes.data, a.ctypes.data, a.ctypes.data, 0.02, -1.0, 0, 0, n=8, stream=0)
+    assert ei.value.code == "E_INVALID"
 
 
 def test_sor_plan_validation_and_no_device():

@@ -1,0 +1,102 @@
+"""GPU parity for Black-Scholes (include/bs.h) through the
+C ABI against the double-precision oracle (oracle/blackscholes.c).  Bar (reading B4): every
+price within 16 eps x the oracle's first-order float32 error scale.  -m gpu only."""
+import numpy as np
+import pytest
+
+import oracle
+from paper_conf_asplos_phothilimthanaara13_b200 import bs, synth
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+EPS32 = 2.0 ** -24
+R, V = synth.BS_RATE, synth.BS_VOL
+
+
+def gpu_price(s, x, t, r=R, v=V, offset=0):
+    n = s.size
+    dev = [torch.empty(n + offset, dtype=torch.float32, device="cuda") for _ in range(5)]
+    for d, a in zip(dev[:3], (s, x, t)):
+        d[offset:] = torch.from_numpy(a)
+    c, p = dev[3], dev[4]
+    c.fill_(float("nan"))
+    p.fill_(float("nan"))
+    bs.price(dev[0][offset:], dev[1][offset:], dev[2][offset:], r, v, c[offset:], p[offset:], n=n)
+    torch.cuda.synchronize()
+    return c[offset:].cpu().numpy(), p[offset:].cpu().numpy()
+
+
+def check(s, x, t, c, p, r=R, v=V):
+    oc, op, scale = oracle.black_scholes(s, x, t, r, v, with_scale=True)
+    assert not np.any(np.isnan(c)) and not np.any(np.isnan(p)), "an output was not written"
+    ec = np.max(np.abs(c - oc) / scale)
+    ep = np.max(np.abs(p - op) / scale)
+    assert ec <= 16 * EPS32 and ep <= 16 * EPS32, (ec / EPS32, ep / EPS32)
+    return ec, ep
+
+
+@pytest.mark.parametrize("n", [1, 3, 4, 1000, 500000, 1000003])
+def test_random_options_within_bound(n):
+    s, x, t = synth.bs_options(n, seed=n)
+    c, p = gpu_price(s, x, t)
+    check(s, x, t, c, p)
+
+
+def test_unaligned_pointers_take_the_scalar_path():
+    s, x, t = synth.bs_options(4099, seed=3)
+    c0, p0 = gpu_price(s, x, t)
+    c1, p1 = gpu_price(s, x, t, offset=1)
+    check(s, x, t, c1, p1)
+    assert np.max(np.abs(c0 - c1)) <= 4 * EPS32 * np.max(np.abs(c0) + s)
+
+
+def test_textbook_example_and_put_call_parity():
+    c, p = gpu_price(np.array([42], np.float32), np.array([40], np.float32), np.array([0.5], np.float32), 0.1, 0.2)
+    assert abs(c[0] - 4.76) <= 0.005 and abs(p[0] - 0.81) <= 0.005
+    s, x, t = synth.bs_options(100000, seed=8)
+    c, p = gpu_price(s, x, t)
+    fwd = s.astype(np.float64) - x.astype(np.float64) * np.exp(-R * t.astype(np.float64))
+    scale = oracle.black_scholes(s, x, t, R, V, with_scale=True)[2]
+    assert np.all(np.abs((c.astype(np.float64) - p) - fwd) <= 32 * EPS32 * scale)
+
+
+def test_other_rates_and_volatilities():
+    s, x, t = synth.bs_options(50000, seed=13)
+    for r, v in ((0.0, 0.1), (0.08, 0.6), (-0.01, 0.25)):
+        c, p = gpu_price(s, x, t, r, v)
+        check(s, x, t, c, p, r, v)
+
+
+def test_host_variant_equals_device_variant():
+    n = (8 << 20) * 2 + 12345                     # three chunks, the last ragged
+    s, x, t = synth.bs_options(n, seed=21)
+    c_dev, p_dev = gpu_price(s, x, t)
+    hs, hx, ht = (torch.from_numpy(a).pin_memory() for a in (s, x, t))
+    hc = torch.empty(n, dtype=torch.float32).pin_memory()
+    hp = torch.empty(n, dtype=torch.float32).pin_memory()
+    bs.price_host(hs, hx, ht, R, V, hc, hp)
+    assert np.array_equal(hc.numpy(), c_dev) and np.array_equal(hp.numpy(), p_dev)
+    idx = np.arange(0, n, 101)
+    check(s[idx], x[idx], t[idx], c_dev[idx], p_dev[idx])
+
+
+def test_bench_size_sampled():
+    """The bench's 2^28 options (5.4 GB of traffic per pass): every 4099th option vs the oracle."""
+    n = 1 << 28
+    s, x, t = synth.bs_options(n, seed=synth.BENCH_SEED_BASE + 50)
+    c, p = gpu_price(s, x, t)
+    idx = np.arange(0, n, 4099)
+    check(s[idx], x[idx], t[idx], c[idx], p[idx])
+    assert np.all(c >= -1e-3) and np.all(p >= -1e-3)             # prices are non-negative (to rounding)
+
+
+def test_errors():
+    a = torch.ones(16, device="cuda")
+    out = torch.empty(16, device="cuda")
+    with pytest.raises(bs.SepconvError) as ei:
+        bs.price(a, a, a, R, 0.0, out, torch.empty(16, device="cuda"))
+    assert ei.value.code == "E_INVALID"
+    with pytest.raises(bs.SepconvError) as ei:
+        bs.price(a, a, a, R, V, a, out)
+    assert ei.value.code == "E_ALIAS"
+    bs.price(a, a, a, R, V, out, torch.empty(16, device="cuda"), n=0)   # no-op
