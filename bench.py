@@ -11,7 +11,8 @@ variant.  At N > 1 (torchrun) the image is split into N row bands, one per GPU, 
 every pass exchanges the (K-1)-row halo with NCCL send/recv inside the C ABI
 (sepconv_run_band); scaling is strong (fixed image).  --workload batch is
 configs[4] (64 x 4096^2, K = 11, images sharded over ranks, no exchange).  --workload
-poisson is the NEXT-3 Poisson2D red-black SOR leg (bench_poisson.py).
+poisson is the NEXT-3 Poisson2D red-black SOR leg (bench_poisson.py), --workload
+blackscholes the NEXT-4 Black-Scholes leg (bench_bs.py).
 
 value = output pixels of the whole job per step / max-over-ranks device time
 (CUDA events, inputs resident in HBM; the 1.07 GB image is larger than the 126 MB
@@ -49,7 +50,7 @@ def parse_args():
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--workload", choices=["image", "batch", "poisson"], default="image")
+    ap.add_argument("--workload", choices=["image", "batch", "poisson", "blackscholes"], default="image")
     ap.add_argument("--widths", default="3,5,7,9,11,13,15,17")
     ap.add_argument("--size", type=int, default=16384, help="image side (image workload)")
     ap.add_argument("--variant", default="auto")
@@ -58,6 +59,7 @@ def parse_args():
     ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle time for the cpu_baseline sample")
     ap.add_argument("--tune-reps", type=int, default=10)
     ap.add_argument("--sor-iters", type=int, default=24, help="poisson workload: iterations per step")
+    ap.add_argument("--options", type=int, default=1 << 28, help="blackscholes workload: options per GPU")
     return ap.parse_args()
 
 
@@ -206,6 +208,9 @@ def main():
     if args.workload == "poisson":
         import bench_poisson
         return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit)
+    if args.workload == "blackscholes":
+        import bench_bs
+        return bench_bs.run(args, peaks, dist_env, ClockSampler, emit)
     if args.impl == "reference":
         return run_reference(args)
 

@@ -12,7 +12,8 @@
  *   B2  the textbook formula: d1 = (ln(S/X) + (r + v^2/2) T) / (v sqrt T), d2 = d1 - v sqrt T,
  *       call = S N(d1) - X e^{-rT} N(d2), put = X e^{-rT} N(-d2) - S N(-d1),
  *       N(x) = erfc(-x / sqrt 2) / 2;
- *   B3  float32 with IEEE-accurate libdevice logf/expf/sqrtf/erfcf (no fast-math);
+ *   B3  float32: libdevice logf/expf/erfcf (no fast-math), the quotient S/X and the
+ *       reciprocal square root on the SFU (~2 ulp each);
  *   B4  tolerance vs the double definition: |g - o| <= 16 eps (S phi(d1) dd + X e^{-rT}
  *       phi(d2) dd + S + X e^{-rT}), eps = 2^-24, dd the conditioning of d1 (oracle).
  * The paper's CPU/GPU work split (25/75 on its laptop) is not built: there

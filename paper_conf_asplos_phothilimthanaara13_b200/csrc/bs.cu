@@ -2,7 +2,7 @@
 // P:1270-1276).
 //
 // One option per entry (reading B1), the textbook formula (B2) in float32 with the
-// accurate libdevice logf / expf / sqrtf / erfcf (B3).  Purely elementwise: 12 B read and
+// accurate libdevice logf / expf / erfcf and SFU reciprocals (B3).  Purely elementwise: 12 B read and
 // 8 B written per option; each thread prices 4 options from 16-byte loads (the scalar
 // path takes unaligned pointers and the ragged tail).  The host variant streams chunks
 // through a two-slot device workspace on two streams so the copy engines overlap.
@@ -20,10 +20,15 @@ namespace bs {
 
 constexpr int kThreads = 256;
 
-__device__ __forceinline__ void price1(float S, float X, float T, float r, float v, float &call, float &put) {
-    const float sq = sqrtf(T);
-    const float vs = v * sq;
-    const float d1 = (logf(S / X) + (r + 0.5f * v * v) * T) / vs;
+// The kernel is issue-bound (ncu: 83% issue-active at 180 instructions per option with IEEE
+// division and sqrt), so the two divisions and the square root use the SFU: 1/(v sqrt T) =
+// rsqrt(T) / v (1/v formed once on the host), sqrt T = T rsqrt(T), S/X = __fdividef.  Each
+// adds ~2 ulp to d1 or to the quotient inside the log, inside the B4 bound.
+__device__ __forceinline__ void price1(float S, float X, float T, float r, float v, float inv_v, float &call,
+                                       float &put) {
+    const float rs = rsqrtf(T);
+    const float vs = v * (T * rs);                      // v sqrt T
+    const float d1 = (logf(__fdividef(S, X)) + (r + 0.5f * v * v) * T) * (rs * inv_v);
     const float d2 = d1 - vs;
     const float disc = X * expf(-r * T);
     const float k = 0.70710678118654752f;             // 1 / sqrt 2
@@ -35,15 +40,15 @@ __device__ __forceinline__ void price1(float S, float X, float T, float r, float
 
 __global__ void __launch_bounds__(kThreads) bs_kernel_vec(const float4 *__restrict__ s, const float4 *__restrict__ x,
                                                           const float4 *__restrict__ t, long long n4, float r, float v,
-                                                          float4 *__restrict__ call, float4 *__restrict__ put) {
+                                                          float inv_v, float4 *__restrict__ call, float4 *__restrict__ put) {
     for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < n4;
          i += static_cast<long long>(gridDim.x) * blockDim.x) {
         const float4 S = __ldcs(s + i), X = __ldcs(x + i), T = __ldcs(t + i);    // streamed once
         float4 c, p;
-        price1(S.x, X.x, T.x, r, v, c.x, p.x);
-        price1(S.y, X.y, T.y, r, v, c.y, p.y);
-        price1(S.z, X.z, T.z, r, v, c.z, p.z);
-        price1(S.w, X.w, T.w, r, v, c.w, p.w);
+        price1(S.x, X.x, T.x, r, v, inv_v, c.x, p.x);
+        price1(S.y, X.y, T.y, r, v, inv_v, c.y, p.y);
+        price1(S.z, X.z, T.z, r, v, inv_v, c.z, p.z);
+        price1(S.w, X.w, T.w, r, v, inv_v, c.w, p.w);
         __stcs(call + i, c);
         __stcs(put + i, p);
     }
@@ -51,11 +56,11 @@ __global__ void __launch_bounds__(kThreads) bs_kernel_vec(const float4 *__restri
 
 __global__ void __launch_bounds__(kThreads) bs_kernel_scalar(const float *__restrict__ s, const float *__restrict__ x,
                                                              const float *__restrict__ t, long long n, float r, float v,
-                                                             float *__restrict__ call, float *__restrict__ put) {
+                                                             float inv_v, float *__restrict__ call, float *__restrict__ put) {
     for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < n;
          i += static_cast<long long>(gridDim.x) * blockDim.x) {
         float c, p;
-        price1(s[i], x[i], t[i], r, v, c, p);
+        price1(s[i], x[i], t[i], r, v, inv_v, c, p);
         call[i] = c;
         put[i] = p;
     }
@@ -88,7 +93,7 @@ static cudaError_t launch(const float *s, const float *x, const float *t, long l
         const long long blocks = std::min<long long>((n4 + kThreads - 1) / kThreads, static_cast<long long>(sms) * 8);
         bs_kernel_vec<<<static_cast<int>(blocks), kThreads, 0, st>>>(
             reinterpret_cast<const float4 *>(s), reinterpret_cast<const float4 *>(x), reinterpret_cast<const float4 *>(t),
-            n4, r, v, reinterpret_cast<float4 *>(call), reinterpret_cast<float4 *>(put));
+            n4, r, v, 1.0f / v, reinterpret_cast<float4 *>(call), reinterpret_cast<float4 *>(put));
         sepconv::g_launches.fetch_add(1, std::memory_order_relaxed);
         done = n4 * 4;
     }
@@ -96,7 +101,7 @@ static cudaError_t launch(const float *s, const float *x, const float *t, long l
         const long long rem = n - done;
         const long long blocks = std::min<long long>((rem + kThreads - 1) / kThreads, static_cast<long long>(sms) * 8);
         bs_kernel_scalar<<<static_cast<int>(blocks), kThreads, 0, st>>>(s + done, x + done, t + done, rem, r, v,
-                                                                        call + done, put + done);
+                                                                        1.0f / v, call + done, put + done);
         sepconv::g_launches.fetch_add(1, std::memory_order_relaxed);
     }
     return cudaGetLastError();
