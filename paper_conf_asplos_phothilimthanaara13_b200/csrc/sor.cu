@@ -174,10 +174,11 @@ struct Wave {
     static constexpr int HL = (2 * T + 3) / 4;       // halo lanes per side
     static constexpr int OUT_LANES = 32 - 2 * HL;
     static constexpr int WOUT = 4 * OUT_LANES;       // split columns written per strip
-    static constexpr int PF = 6;                     // rows prefetched ahead of the wavefront
-    static constexpr int RDU = 8;                    // u ring rows (>= PF + 1), one mbarrier each
-    // b ring rows: row r - 2T (black_T at step r) must survive until row r + PF lands
-    static constexpr int RDB = (2 * T + PF + 1 <= 16) ? 16 : 32;
+    static constexpr int PF = 3;                     // rows prefetched ahead of the wavefront
+    static constexpr int RDU = 4;                    // u ring rows (>= PF + 1), one mbarrier each
+    // b ring rows: row r - 2T (black_T at step r) must survive until row r + PF lands;
+    // 12 rows (T <= 4) keep a 4-warp CTA at 64 KB: 3 CTAs (12 warps) per SM
+    static constexpr int RDB = (2 * T + PF + 1 <= 12) ? 12 : (2 * T + PF + 1 <= 16 ? 16 : 32);
     static constexpr int WARP_FLOATS = 128 * (2 * RDU + 2 * RDB);
     static constexpr size_t SMEM = static_cast<size_t>(kWaveWarps) * (WARP_FLOATS * 4 + RDU * 8);
     static_assert(2 * T + PF + 1 <= RDB, "b ring too shallow");
