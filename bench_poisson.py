@@ -4,10 +4,10 @@ Fig. 8).  Not the headline metric (BASELINE.json names SeparableConvolutio
 
 A "step" = `--sor-iters` red-black iterations of an N x N grid (default 16384^2, 24
 iterations) with the tuned variant, inputs resident in HBM (split once before timing).
-value = cell-updates of the whole job per second (N*N*iters per rank / max-over-ranks device
-time).  N > 1: every rank solves its own grid (independent problems, weak scaling; the
-per-iteration halo exchange of a row-band split is not built -- DESIGN.md section 11).
-e2e = sor_solve_host with pinned host buffers (x, b in; u out) per step.  cpu_baseline =
+value = cell-updates of the whole job per second (N*N*iters / max-over-ranks device time).
+N > 1: the grid is split into row bands (sor_band), one per rank, with 2T ghost rows
+refreshed by NCCL send/recv after every wavefront pass of depth T (sor_band_iterate):
+strong scaling.  e2e (N = 1) = sor_solve_host with pinned host buffers (x, b in; u out).  cpu_baseline =
 the double-precision oracle (oracle/poisson.c) on a bounded sub-grid sample."""
 from __future__ import annotations
 
@@ -73,15 +73,44 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
     peak_gbs, peak_src = peaks_fn()
     n = args.size
     iters = args.sor_iters
-    x, b = synth.poisson_problem(n, n, seed=synth.BENCH_SEED_BASE + 40 + rank, guess="uniform")
+    x, b = synth.poisson_problem(n, n, seed=synth.BENCH_SEED_BASE + 40, guess="uniform")
     omega = synth.omega_opt(n, n)
-    dx, db = torch.from_numpy(x).to(dev), torch.from_numpy(b).to(dev)
     stream = torch.cuda.current_stream(dev)
-    p = sor.SorPlan(n, n)
-    variant_id, depth = p.tune(iters_hint=iters, reps=3)
+    if world > 1:
+        # one grid in row bands: every rank must run the same passes (same depth), so rank
+        # 0's tuned choice is broadcast; halo = 2 x depth ghost rows, exchanged by NCCL
+        probe = sor.SorPlan(max(64, n // world), n)
+        choice = torch.tensor(list(probe.tune(iters_hint=iters, reps=3)), dtype=torch.int64, device=dev)
+        probe.close()
+        dist.broadcast(choice, 0)
+        variant_id, depth = int(choice[0]), int(choice[1])
+        if variant_id == sor.SOR_HALF:
+            depth = 1
+        halo = 2 * depth
+        r0, rows, a0, arows = sor.band(n, world, rank, halo)
+        raw = sc.nccl_unique_id() if rank == 0 else bytes(sc.NCCL_ID_BYTES)
+        t = torch.tensor(list(raw), dtype=torch.uint8, device=dev)
+        dist.broadcast(t, 0)
+        p = sor.SorPlan(arows, n)
+        p.set_depth(depth)
+        p.comm_init(bytes(t.cpu().tolist()), world, rank, halo)
+        dx = torch.from_numpy(np.ascontiguousarray(x[a0:a0 + arows])).to(dev)
+        db = torch.from_numpy(np.ascontiguousarray(b[a0:a0 + arows])).to(dev)
+        vname = "half" if variant_id == sor.SOR_HALF else "wave"
+
+        def step():
+            p.band_iterate(omega, iters, vname, stream)
+    else:
+        p = sor.SorPlan(n, n)
+        variant_id, depth = p.tune(iters_hint=iters, reps=3)
+        dx, db = torch.from_numpy(x).to(dev), torch.from_numpy(b).to(dev)
+        rows = n
+
+        def step():
+            p.iterate(omega, iters, "auto", stream)
     p.load(dx, db)
     for _ in range(max(args.warmup, 0)):
-        p.iterate(omega, iters, "auto", stream)
+        step()
     torch.cuda.synchronize()
     if dist:
         dist.barrier()
@@ -90,10 +119,10 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
     with ClockSampler(local) as clk:
         torch.cuda.synchronize()
         torch.cuda.nvtx.range_push("sepconv_timed")
-        for s in range(args.steps):
-            ev[s][0].record(stream)
-            p.iterate(omega, iters, "auto", stream)
-            ev[s][1].record(stream)
+        for i in range(args.steps):
+            ev[i][0].record(stream)
+            step()
+            ev[i][1].record(stream)
         torch.cuda.nvtx.range_pop()
         torch.cuda.synchronize()
     launches = sc.launch_count() - launches0
@@ -102,7 +131,7 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
         t = torch.tensor([ms], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         ms = float(t[0])
-    cells = n * n * iters * world
+    cells = n * n * iters                       # the whole grid (strong scaling over row bands)
     value = cells / (ms * 1e-3) / 1e6
     if variant_id == sor.SOR_HALF:
         kern, byts, launches_per = "sor_half_kernel", 16.0 * n * n, 2
@@ -111,6 +140,7 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
         kern, byts, launches_per = f"sor_wave_kernel<{depth}>", 12.0 * n * n, 1
         algo = f"12 B per cell per pass of {depth} iterations (u and b read once, u written once)"
     passes = iters if variant_id == sor.SOR_HALF else -(-iters // depth)
+    byts = byts * rows / n                      # this rank's share of the grid
     achieved = byts * passes / (ms * 1e-3) / 1e9
     roofline = {"bound": "hbm", "kernel": kern, "achieved": achieved, "peak": peak_gbs, "unit": "GB/s",
                 "frac": achieved / peak_gbs, "traffic": None, "peak_source": peak_src,
@@ -120,7 +150,7 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
                         "~98% of the measured copy but moves 16 B per cell-iteration"}
 
     e2e = None
-    if not args.no_e2e:
+    if not args.no_e2e and world == 1:
         hx, hb = torch.from_numpy(x).pin_memory(), torch.from_numpy(b).pin_memory()
         hu = torch.empty((n, n), dtype=torch.float32).pin_memory()
         p.solve_host(hx, hb, hu, omega, iters, "auto", stream)
@@ -143,13 +173,14 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
         cpu = _oracle_sample(args.cpu_seconds)
     if rank == 0:
         emit({"metric": METRIC, "value": value, "unit": "Mcell-it/s", "n_gpus": world, "steps": args.steps,
-              "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
+              "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f32", "data": "synthetic",
               "config": {"workload": f"Poisson2D red-black SOR, {n}x{n} float32 grid, {iters} iterations per step",
                          "grid": [n, n], "iters_per_step": iters, "omega": omega,
                          "variant": "auto (tuned): " + ("half" if variant_id == sor.SOR_HALF else f"wave depth {depth}"),
                          "l2": "grid larger than L2" if 6 * n * n * 4 > 126e6 else "L2-resident (the paper's 2048^2)",
-                         "parallelism": f"independent grids x{world}" if world > 1 else "1 GPU"},
+                         "parallelism": (f"row bands x{world}, {2 * depth}-row ghost exchange per pass (NCCL)"
+                                         if world > 1 else "1 GPU")},
               "gcell_it_s": value / 1e3, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
               "gpu_launches": int(launches), "launches_per_pass": launches_per, "clocks": clk.summary()})
     p.close()

@@ -94,6 +94,29 @@ sepconv_status_t sor_tune(sor_plan_t plan, int iters_hint, int reps, int *varian
  * tests and measurements; E_INVALID outside 0..8. */
 sepconv_status_t sor_set_depth(sor_plan_t plan, int depth);
 
+/* ---- row bands across GPUs (one process per GPU) ----------------------------------
+ * Band g of G owns grid rows [row0, row0 + rows), row0 = 2 floor(g N / 2G) (even: the
+ * colouring P3 is the same in band and grid coordinates); it is planned as a grid of
+ * alloc_rows rows starting at grid row alloc_row0: `halo` ghost rows above and below where
+ * a neighbour exists.  The caller loads x and b for those alloc rows (sor_load) and stores
+ * the result (sor_store: the owned rows are rows [row0 - alloc_row0, + rows)).
+ * E_INVALID when a band is thinner than the halo or the halo is odd. */
+sepconv_status_t sor_band(int64_t n, int nbands, int g, int halo, int64_t *row0, int64_t *rows, int64_t *alloc_row0,
+                          int64_t *alloc_rows);
+
+/* Make `plan` (planned with alloc_rows x M) band `rank` of `nranks` with `halo` ghost rows
+ * (even, >= 2).  id: a sepconv_nccl_unique_id() shared by all ranks (NCCL communicator,
+ * reference-counted per id), or NULL for external mode, where the caller refreshes the
+ * ghost rows between calls (tests on one GPU). */
+sepconv_status_t sor_comm_init(sor_plan_t plan, const unsigned char *id, int nranks, int rank, int halo);
+
+/* `iters` iterations of the band in passes of depth T <= halo/2 (SOR_WAVE) or 1 (SOR_HALF);
+ * after every pass the ghost rows of both colours are exchanged with the neighbours by
+ * NCCL grouped send/recv on `stream` (skipped in external mode).  The owned rows equal the
+ * single-GPU result bit for bit. */
+sepconv_status_t sor_band_iterate(sor_plan_t plan, float omega, int iters, sor_variant_t variant,
+                                  sepconv_stream_t stream);
+
 void sor_destroy(sor_plan_t plan);                  /* NULL-safe; waits for the device */
 
 #ifdef __cplusplus

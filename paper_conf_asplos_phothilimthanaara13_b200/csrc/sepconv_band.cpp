@@ -22,28 +22,7 @@
 
 using namespace sepconv;
 
-namespace {
-
-// the subset of the NCCL ABI we use (stable since NCCL 2.7)
-typedef int nccl_result_t;
-typedef void *nccl_comm_t;
-struct nccl_unique_id_t {
-    char internal[SEPCONV_NCCL_ID_BYTES];
-};
-constexpr int kNcclFloat32 = 7;
-
-struct NcclApi {
-    bool ok = false;
-    std::string why;
-    nccl_result_t (*GetUniqueId)(nccl_unique_id_t *) = nullptr;
-    nccl_result_t (*CommInitRank)(nccl_comm_t *, int, nccl_unique_id_t, int) = nullptr;
-    nccl_result_t (*CommDestroy)(nccl_comm_t) = nullptr;
-    nccl_result_t (*Send)(const void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
-    nccl_result_t (*Recv)(void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
-    nccl_result_t (*GroupStart)() = nullptr;
-    nccl_result_t (*GroupEnd)() = nullptr;
-    const char *(*GetErrorString)(nccl_result_t) = nullptr;
-};
+namespace sepconv {
 
 NcclApi &nccl() {
     static NcclApi api;
@@ -78,6 +57,10 @@ NcclApi &nccl() {
     return api;
 }
 
+}  // namespace sepconv
+
+namespace {
+
 // Communicators are shared by every plan of the process that is initialised with the same
 // unique id, rank and size (e.g. one plan per kernel width over the same row bands): the
 // first sepconv_comm_init creates it collectively, later ones take a reference.
@@ -101,12 +84,51 @@ void release_comm(void *comm) {
     }
 }
 
+}  // namespace
+
+namespace sepconv {
 sepconv_status_t nccl_fail(nccl_result_t r, const char *what) {
     NcclApi &a = nccl();
     return fail(SEPCONV_E_NCCL, "%s: %s", what, a.GetErrorString ? a.GetErrorString(r) : "error");
 }
 
-}  // namespace
+// A communicator for (id, nranks, rank) on `device`, created collectively on first use and
+// reference-counted; release with comm_release.
+sepconv_status_t comm_acquire(const unsigned char *id, int nranks, int rank, int device, void **out) {
+    NcclApi &a = nccl();
+    if (!a.ok) return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
+    const std::string key(reinterpret_cast<const char *>(id), SEPCONV_NCCL_ID_BYTES);
+    std::lock_guard<std::mutex> lock(g_comm_mu);
+    auto it = g_comms.find(key);
+    if (it != g_comms.end()) {
+        if (it->second.nranks != nranks || it->second.rank != rank || it->second.device != device)
+            return fail(SEPCONV_E_INVALID, "NCCL id already used with a different rank, size or device");
+        ++it->second.refs;
+        *out = it->second.comm;
+        return SEPCONV_OK;
+    }
+    nccl_unique_id_t u;
+    std::memcpy(u.internal, id, SEPCONV_NCCL_ID_BYTES);
+    nccl_comm_t comm = nullptr;
+    int prev = -1;
+    cudaGetDevice(&prev);
+    cudaSetDevice(device);
+    nccl_result_t r = a.CommInitRank(&comm, nranks, u, rank);
+    if (prev >= 0) cudaSetDevice(prev);
+    if (r != 0) return nccl_fail(r, "ncclCommInitRank");
+    SharedComm sc;
+    sc.comm = comm;
+    sc.nranks = nranks;
+    sc.rank = rank;
+    sc.refs = 1;
+    sc.device = device;
+    g_comms[key] = sc;
+    *out = comm;
+    return SEPCONV_OK;
+}
+
+void comm_release(void *comm) { release_comm(comm); }
+}  // namespace sepconv
 
 void sepconv_comm_destroy_internal(sepconv_plan_t plan) {
     if (plan->comm) release_comm(plan->comm);
@@ -171,39 +193,9 @@ sepconv_status_t sepconv_comm_init(sepconv_plan_t plan, const unsigned char id[S
         return SEPCONV_OK;
     }
     plan->band_external = false;
-    NcclApi &a = nccl();
-    if (!a.ok) {
-        if (prev >= 0) cudaSetDevice(prev);
-        return fail(SEPCONV_E_NCCL, "%s", a.why.c_str());
-    }
-    const std::string key(reinterpret_cast<const char *>(id), SEPCONV_NCCL_ID_BYTES);
-    std::lock_guard<std::mutex> lock(g_comm_mu);
-    auto it = g_comms.find(key);
-    if (it != g_comms.end()) {
-        if (it->second.nranks != nranks || it->second.rank != rank || it->second.device != plan->dev.device) {
-            if (prev >= 0) cudaSetDevice(prev);
-            return fail(SEPCONV_E_INVALID, "NCCL id already used with a different rank, size or device");
-        }
-        ++it->second.refs;
-        plan->comm = it->second.comm;
-        if (prev >= 0) cudaSetDevice(prev);
-        return SEPCONV_OK;
-    }
-    nccl_unique_id_t u;
-    std::memcpy(u.internal, id, SEPCONV_NCCL_ID_BYTES);
-    nccl_comm_t comm = nullptr;
-    nccl_result_t r = a.CommInitRank(&comm, nranks, u, rank);
+    sepconv_status_t st = comm_acquire(id, nranks, rank, plan->dev.device, &plan->comm);
     if (prev >= 0) cudaSetDevice(prev);
-    if (r != 0) return nccl_fail(r, "ncclCommInitRank");
-    SharedComm sc;
-    sc.comm = comm;
-    sc.nranks = nranks;
-    sc.rank = rank;
-    sc.refs = 1;
-    sc.device = plan->dev.device;
-    g_comms[key] = sc;
-    plan->comm = comm;
-    return SEPCONV_OK;
+    return st;
 }
 
 sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const float *kernel, float *out_band,

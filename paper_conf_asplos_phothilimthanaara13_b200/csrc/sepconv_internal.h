@@ -110,4 +110,30 @@ sepconv_status_t ensure_buf(sepconv_plan_t plan);
 }  // namespace sepconv
 
 void sepconv_comm_destroy_internal(sepconv_plan_t plan);   // sepconv_band.cpp
+
+// ---- NCCL, loaded at run time (sepconv_band.cpp); shared by the row-band paths ----------
+namespace sepconv {
+typedef int nccl_result_t;                 // the subset of the NCCL ABI we use (stable since 2.7)
+typedef void *nccl_comm_t;
+struct nccl_unique_id_t {
+    char internal[SEPCONV_NCCL_ID_BYTES];
+};
+constexpr int kNcclFloat32 = 7;
+struct NcclApi {
+    bool ok = false;
+    std::string why;
+    nccl_result_t (*GetUniqueId)(nccl_unique_id_t *) = nullptr;
+    nccl_result_t (*CommInitRank)(nccl_comm_t *, int, nccl_unique_id_t, int) = nullptr;
+    nccl_result_t (*CommDestroy)(nccl_comm_t) = nullptr;
+    nccl_result_t (*Send)(const void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
+    nccl_result_t (*Recv)(void *, size_t, int, int, nccl_comm_t, cudaStream_t) = nullptr;
+    nccl_result_t (*GroupStart)() = nullptr;
+    nccl_result_t (*GroupEnd)() = nullptr;
+    const char *(*GetErrorString)(nccl_result_t) = nullptr;
+};
+NcclApi &nccl();
+sepconv_status_t nccl_fail(nccl_result_t r, const char *what);
+sepconv_status_t comm_acquire(const unsigned char *id, int nranks, int rank, int device, void **out);
+void comm_release(void *comm);
+}  // namespace sepconv
 void sepconv_seed_from_cache(sepconv_plan_t plan);         // sepconv_tune.cpp

@@ -405,6 +405,10 @@ struct sor_plan_s {
     int variant = -1, depth = 0;     // tuned (variant < 0: untuned)
     int forced_depth = 0;
     int wave_occ[sor::kMaxDepth + 1] = {};
+    // row bands (sor_comm_init): this plan holds rows [row0 - h_top, row1 + h_bot) of the grid
+    bool band = false, band_external = false;
+    void *comm = nullptr;
+    int nranks = 1, rank = 0, halo = 0, h_top = 0, h_bot = 0;
 };
 
 namespace {
@@ -559,6 +563,7 @@ sepconv_status_t sor_plan(int64_t n, int64_t m, sor_plan_t *out) {
 void sor_destroy(sor_plan_t plan) {
     if (!plan) return;
     cudaDeviceSynchronize();
+    if (plan->comm) sepconv::comm_release(plan->comm);
     cudaFree(plan->buf);
     delete plan;
 }
@@ -683,6 +688,103 @@ sepconv_status_t sor_set_depth(sor_plan_t plan, int depth) {
     if (sepconv_status_t s = check_plan(plan)) return s;
     if (depth < 0 || depth > sor::kMaxDepth) return fail(SEPCONV_E_INVALID, "depth %d outside 0..%d", depth, sor::kMaxDepth);
     plan->forced_depth = depth;
+    return SEPCONV_OK;
+}
+
+// ---- row bands across GPUs -------------------------------------------------------------
+// Owned rows of band g: [r_g, r_{g+1}) with r_g = 2 floor(g N / 2G) (even, so every band's
+// first local row has an even global index and the red/black colouring of P3 is the same in
+// local and global coordinates); r_G = N.  A band plan holds its owned rows plus `halo` ghost
+// rows on each side that has a neighbour.  A pass of depth T leaves the owned rows exact when
+// halo >= 2T: the ghost rows are treated as fixed, and the error that introduces moves one
+// row inward per half-sweep.
+sepconv_status_t sor_band(int64_t n, int nbands, int g, int halo, int64_t *row0, int64_t *rows, int64_t *alloc_row0,
+                          int64_t *alloc_rows) {
+    if (n < 1 || nbands < 1 || g < 0 || g >= nbands) return fail(SEPCONV_E_INVALID, "band %d of %d", g, nbands);
+    if (halo < 0 || (halo & 1)) return fail(SEPCONV_E_INVALID, "halo %d must be even and >= 0", halo);
+    const int64_t r0 = 2 * ((static_cast<int64_t>(g) * n) / (2LL * nbands));
+    const int64_t r1 = g + 1 == nbands ? n : 2 * ((static_cast<int64_t>(g + 1) * n) / (2LL * nbands));
+    if (nbands > 1 && (r1 - r0) < std::max(halo, 1))
+        return fail(SEPCONV_E_INVALID, "band %d has %lld rows, fewer than the %d-row halo", g, (long long)(r1 - r0), halo);
+    const int64_t a0 = g > 0 ? r0 - halo : r0;
+    const int64_t a1 = g + 1 < nbands ? r1 + halo : r1;
+    if (a0 < 0 || a1 > n) return fail(SEPCONV_E_INVALID, "halo %d larger than the neighbouring band", halo);
+    if (row0) *row0 = r0;
+    if (rows) *rows = r1 - r0;
+    if (alloc_row0) *alloc_row0 = a0;
+    if (alloc_rows) *alloc_rows = a1 - a0;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_comm_init(sor_plan_t plan, const unsigned char *id, int nranks, int rank, int halo) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (nranks < 1 || rank < 0 || rank >= nranks) return fail(SEPCONV_E_INVALID, "rank %d of %d", rank, nranks);
+    if (halo < 2 || (halo & 1)) return fail(SEPCONV_E_INVALID, "halo %d must be even and >= 2", halo);
+    const int h_top = rank > 0 ? halo : 0, h_bot = rank + 1 < nranks ? halo : 0;
+    if (plan->n - h_top - h_bot < halo && nranks > 1)
+        return fail(SEPCONV_E_INVALID, "band of %lld rows cannot hold %d owned rows plus its ghost rows",
+                    (long long)plan->n, halo);
+    if (plan->comm) {
+        sepconv::comm_release(plan->comm);
+        plan->comm = nullptr;
+    }
+    plan->band = true;
+    plan->band_external = id == nullptr;
+    plan->nranks = nranks;
+    plan->rank = rank;
+    plan->halo = halo;
+    plan->h_top = h_top;
+    plan->h_bot = h_bot;
+    if (id && nranks > 1) return sepconv::comm_acquire(id, nranks, rank, plan->device, &plan->comm);
+    return SEPCONV_OK;
+}
+
+// refresh the ghost rows of the current iterate from the neighbours' owned rows (both colours)
+static sepconv_status_t band_exchange(sor_plan_t plan, cudaStream_t st) {
+    if (plan->band_external || plan->nranks == 1 || !plan->comm) return SEPCONV_OK;
+    sepconv::NcclApi &a = sepconv::nccl();
+    const size_t cnt = static_cast<size_t>(plan->halo) * plan->ldh;
+    const int64_t n = plan->n, ldh = plan->ldh;
+    sepconv::nccl_comm_t comm = plan->comm;
+    sepconv::nccl_result_t r = a.GroupStart();
+    for (int c = 0; c < 2 && r == 0; ++c) {
+        float *buf = plan->u[plan->cur][c];
+        if (plan->rank > 0) {               // first owned rows up, top ghost rows from above
+            if (r == 0) r = a.Send(buf + plan->h_top * ldh, cnt, sepconv::kNcclFloat32, plan->rank - 1, comm, st);
+            if (r == 0) r = a.Recv(buf, cnt, sepconv::kNcclFloat32, plan->rank - 1, comm, st);
+        }
+        if (plan->rank + 1 < plan->nranks) {  // last owned rows down, bottom ghost rows from below
+            if (r == 0) r = a.Send(buf + (n - plan->h_bot - plan->halo) * ldh, cnt, sepconv::kNcclFloat32, plan->rank + 1,
+                                   comm, st);
+            if (r == 0) r = a.Recv(buf + (n - plan->halo) * ldh, cnt, sepconv::kNcclFloat32, plan->rank + 1, comm, st);
+        }
+    }
+    sepconv::nccl_result_t r2 = a.GroupEnd();
+    if (r != 0) return sepconv::nccl_fail(r, "ncclSend/ncclRecv (SOR ghost rows)");
+    if (r2 != 0) return sepconv::nccl_fail(r2, "ncclGroupEnd");
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sor_band_iterate(sor_plan_t plan, float omega, int iters, sor_variant_t variant,
+                                  sepconv_stream_t stream) {
+    if (sepconv_status_t s = check_plan(plan)) return s;
+    if (!plan->band) return fail(SEPCONV_E_INVALID, "sor_comm_init has not been called on this plan");
+    if (!(omega > 0.f && omega < 2.f)) return fail(SEPCONV_E_INVALID, "omega %g outside (0, 2)", (double)omega);
+    if (iters < 0) return fail(SEPCONV_E_INVALID, "iters %d < 0", iters);
+    if (variant < SOR_HALF || variant > SOR_AUTO) return fail(SEPCONV_E_INVALID, "unknown variant %d", (int)variant);
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    int v = variant, depth = plan->forced_depth;
+    if (v == SOR_AUTO) v = plan->variant >= 0 ? plan->variant : SOR_WAVE;
+    if (depth == 0) depth = plan->depth > 0 ? plan->depth : kDefaultDepth;
+    depth = std::max(1, std::min(depth, plan->halo / 2));           // owned rows exact after each pass
+    while (iters > 0) {
+        const int T = v == SOR_HALF ? 1 : std::min(iters, depth);
+        sepconv_status_t s = v == SOR_HALF ? half_iterations(plan, omega, 1, st) : wave_iterations(plan, omega, T, T, st);
+        if (s != SEPCONV_OK) return s;
+        s = band_exchange(plan, st);
+        if (s != SEPCONV_OK) return s;
+        iters -= T;
+    }
     return SEPCONV_OK;
 }
 

@@ -30,6 +30,9 @@ def lib() -> ctypes.CDLL:
             "sor_buffers": (I, [P, pP, pP, pP, pP, pI64]),
             "sor_tune": (I, [P, I, I, pI, pI]),
             "sor_set_depth": (I, [P, I]),
+            "sor_band": (I, [I64, I, I, I, pI64, pI64, pI64, pI64]),
+            "sor_comm_init": (I, [P, ctypes.c_char_p, I, I, I]),
+            "sor_band_iterate": (I, [P, F, I, I, P]),
             "sor_destroy": (None, [P]),
         }
         for name, (res, args) in sig.items():
@@ -42,7 +45,14 @@ def lib() -> ctypes.CDLL:
 
 def exported_symbols():
     return ["sor_plan", "sor_load", "sor_iterate", "sor_store", "sor_solve", "sor_solve_host", "sor_buffers",
-            "sor_tune", "sor_set_depth", "sor_destroy"]
+            "sor_tune", "sor_set_depth", "sor_band", "sor_comm_init", "sor_band_iterate", "sor_destroy"]
+
+
+def band(n: int, nbands: int, g: int, halo: int):
+    """sor_band: (row0, rows, alloc_row0, alloc_rows) of band g of nbands."""
+    vals = [ctypes.c_int64() for _ in range(4)]
+    _check(lib().sor_band(int(n), int(nbands), int(g), int(halo), *[ctypes.byref(v) for v in vals]), "sor_band")
+    return tuple(int(v.value) for v in vals)
 
 
 def _variant(v) -> int:
@@ -110,6 +120,14 @@ class SorPlan:
 
     def set_depth(self, depth: int):
         _check(lib().sor_set_depth(self._h, int(depth)), "sor_set_depth")
+
+    def comm_init(self, unique_id: bytes | None, nranks: int, rank: int, halo: int):
+        """Band `rank` of `nranks` with `halo` ghost rows; unique_id=None = external mode."""
+        _check(lib().sor_comm_init(self._h, unique_id, int(nranks), int(rank), int(halo)), "sor_comm_init")
+
+    def band_iterate(self, omega: float, iters: int, variant="auto", stream=None):
+        _check(lib().sor_band_iterate(self._h, float(omega), int(iters), _variant(variant), _stream(stream)),
+               "sor_band_iterate")
 
 
 __all__ = ["SorPlan", "SOR_HALF", "SOR_WAVE", "SOR_AUTO", "SepconvError", "exported_symbols", "lib"]

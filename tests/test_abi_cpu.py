@@ -31,7 +31,7 @@ def test_library_exports_every_sor_symbol():
     hdr = open(os.path.join(ROOT, "include", "sor.h")).read()
     declared = sorted(set(re.findall(r"\b(sor_[a-z_]+)\s*\(", hdr)))
     L = sor.lib()
-    assert len(declared) == 10
+    assert len(declared) == 13
     for name in declared:
         assert hasattr(L, name), name
     assert sorted(sor.exported_symbols()) == declared
@@ -133,3 +133,24 @@ def test_band_rejects_thin_bands():
 
 def test_band_single_gpu_is_whole_image():
     assert sc.band(100, 7, 1, 0) == (0, 94, 100, 100)
+
+
+@pytest.mark.parametrize("n,G,halo", [(16384, 8, 8), (2048, 2, 6), (101, 3, 4), (1000, 7, 2), (64, 1, 8)])
+def test_sor_band_partition(n, G, halo):
+    covered = 0
+    for g in range(G):
+        r0, rows, a0, arows = sor.band(n, G, g, halo)
+        assert r0 % 2 == 0 and a0 % 2 == 0                # colouring is band-invariant
+        assert r0 == covered
+        covered += rows
+        assert a0 == (r0 - halo if g > 0 else r0)
+        assert a0 + arows == (r0 + rows + halo if g < G - 1 else n)
+        assert rows >= (halo if G > 1 else 1)
+    assert covered == n
+
+
+def test_sor_band_rejects_thin_bands_and_odd_halos():
+    with pytest.raises(sc.SepconvError):
+        sor.band(40, 8, 0, 8)
+    with pytest.raises(sc.SepconvError):
+        sor.band(400, 2, 0, 3)

@@ -170,3 +170,72 @@ def test_sampled_blocks_at_bench_size():
         bottom = h if i0 + h == n else h - margin
         right = w if j0 + w == m else w - margin
         assert np.array_equal(got[i0 + top:i0 + bottom, j0 + left:j0 + right], want[top:bottom, left:right]), (i0, j0)
+
+
+# ---- row bands on one GPU: the band path of sor_band_iterate with the ghost-row exchange
+# ---- done by the test (external mode); NCCL itself with one rank --------------------------
+def _rows_view(ptr, ldh, r0, nrows):
+    return torch.as_tensor(_Raw(int(ptr) + 4 * r0 * ldh, nrows, ldh), device="cuda")
+
+
+@pytest.mark.parametrize("G,halo,variant", [(2, 6, "wave"), (3, 8, "wave"), (4, 2, "half"), (3, 4, "wave")])
+def test_bands_external_exchange_equal_whole_grid(G, halo, variant):
+    N, M, iters = 301, 517, 9
+    x, b = synth.poisson_problem(N, M, seed=55, guess="uniform")
+    omega = synth.omega_opt(N, M)
+    want = gpu_solve(x, b, omega, iters, variant, depth=max(1, halo // 2))
+    bands = []
+    for g in range(G):
+        r0, rows, a0, arows = sor.band(N, G, g, halo)
+        p = sor.SorPlan(arows, M)
+        p.set_depth(max(1, halo // 2))
+        p.load(_dev(x[a0:a0 + arows]), _dev(b[a0:a0 + arows]))
+        p.comm_init(None, G, g, halo)
+        bands.append((p, r0, rows, a0, arows))
+    T = 1 if variant == "half" else halo // 2
+    left = iters
+    while left > 0:
+        t = min(T, left)
+        for p, *_ in bands:
+            p.band_iterate(omega, t, variant)
+        torch.cuda.synchronize()
+        # the exchange a NCCL run does: neighbours' first/last owned rows into the ghost rows
+        views = []
+        for p, r0, rows, a0, arows in bands:
+            (ur, ub, _, _), ldh = p.buffers()
+            views.append((ur, ub, ldh, r0 - a0, a0 + arows - (r0 + rows), arows))
+        for g in range(G):
+            ur, ub, ldh, h_top, h_bot, n = views[g]
+            for c in range(2):
+                mine = (ur, ub)[c]
+                if g > 0:
+                    pur, pub, _, ph_top, ph_bot, pn = views[g - 1]
+                    _rows_view(mine, ldh, 0, halo).copy_(_rows_view((pur, pub)[c], ldh, pn - ph_bot - halo, halo))
+                if g < G - 1:
+                    nur, nub, _, nh_top, _, _ = views[g + 1]
+                    _rows_view(mine, ldh, n - halo, halo).copy_(_rows_view((nur, nub)[c], ldh, nh_top, halo))
+        torch.cuda.synchronize()
+        left -= t
+    got = []
+    for p, r0, rows, a0, arows in bands:
+        u = torch.full((arows, M), float("nan"), device="cuda")
+        p.store(u)
+        torch.cuda.synchronize()
+        got.append(u[r0 - a0:r0 - a0 + rows].cpu().numpy())
+    assert np.array_equal(np.concatenate(got, 0), want)
+
+
+def test_band_nccl_single_rank_equals_plain():
+    from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+    N, M = 130, 250
+    x, b = synth.poisson_problem(N, M, seed=3, guess="uniform")
+    want = gpu_solve(x, b, 1.6, 8, "wave", depth=4)
+    p = sor.SorPlan(N, M)
+    p.set_depth(4)
+    p.load(_dev(x), _dev(b))
+    p.comm_init(sc.nccl_unique_id(), 1, 0, 8)
+    p.band_iterate(1.6, 8, "wave")
+    u = torch.empty((N, M), device="cuda")
+    p.store(u)
+    torch.cuda.synchronize()
+    assert np.array_equal(u.cpu().numpy(), want)
