@@ -264,7 +264,12 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
     const int n = p.n;
     const long long ldh = p.ldh;
     const unsigned nm2 = static_cast<unsigned>(n - 2);                  // row rho is interior iff rho-1 < n-2
-    uint32_t c = 0;                                                      // rows this warp has consumed
+    // row counter of this warp's rings.  The first steps of a segment read b slots of rows
+    // above the segment (counter c - 2T .. c - 1; their values only feed rows that are never
+    // written), so the counter starts past 2T: with RDB not a power of two a wrapped unsigned
+    // counter would alias a slot the prologue is filling.  A multiple of 2 RDU keeps the
+    // mbarrier phase parity (counter / RDU) & 1 at 0 for each barrier's first phase.
+    uint32_t c = 2 * RDU * ((2 * T + 2 * RDU) / (2 * RDU));
 
     for (long long item = gw; item < p.items; item += nw) {
         const int strip = static_cast<int>(item % p.nstrips);
