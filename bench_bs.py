@@ -8,12 +8,16 @@ price their own shard: no exchange, weak scaling).  e2e = bs_price_host on pinne
 buffers.  cpu_baseline = the double oracle on a bounded sample."""
 from __future__ import annotations
 
+import json
+import os
 import statistics
 import time
 
 import numpy as np
 
 from paper_conf_asplos_phothilimthanaara13_b200 import synth
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
 
 METRIC = "Black-Scholes European options priced per second (Moptions/s)"
 
@@ -96,8 +100,13 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
     value = n * world / (ms * 1e-3) / 1e6
     byts = 20.0 * n
     achieved = byts / (ms * 1e-3) / 1e9
+    traffic = None                       # ncu DRAM read + write bytes of one launch (profiles/traffic.json)
+    try:
+        traffic = json.load(open(os.path.join(ROOT, "profiles", "traffic.json"))).get(f"bs_kernel_vec:n{n}")
+    except Exception:
+        traffic = None
     roofline = {"bound": "hbm", "kernel": "bs_kernel_vec", "achieved": achieved, "peak": peak_gbs, "unit": "GB/s",
-                "frac": achieved / peak_gbs, "traffic": None, "peak_source": peak_src,
+                "frac": achieved / peak_gbs, "traffic": traffic, "peak_source": peak_src,
                 "algorithmic_bytes_per_launch": byts, "algorithmic": "20 B per option (S, X, T read; call, put written)"}
     e2e = None
     if not args.no_e2e:

@@ -12,8 +12,10 @@
  *   B2  the textbook formula: d1 = (ln(S/X) + (r + v^2/2) T) / (v sqrt T), d2 = d1 - v sqrt T,
  *       call = S N(d1) - X e^{-rT} N(d2), put = X e^{-rT} N(-d2) - S N(-d1),
  *       N(x) = erfc(-x / sqrt 2) / 2;
- *   B3  float32: libdevice logf/expf/erfcf (no fast-math), the quotient S/X and the
- *       reciprocal square root on the SFU (~2 ulp each);
+ *   B3  float32, every transcendental one SFU instruction (ftz): ln(S/X) = ln2 lg2(S rcp X),
+ *       e^{-rT} = ex2(-rT log2e), 1/(v sqrt T) = rsqrt(T)/v (a few ulp each);
+ *   B5  N(d) and 1 - N(d) from one tail e = erfc(|d|/sqrt 2)/2, erfc the Chebyshev fit of
+ *       Numerical Recipes 6.2 "erfcc" (fractional error < 1.2e-7);
  *   B4  tolerance vs the double definition: |g - o| <= 16 eps (S phi(d1) dd + X e^{-rT}
  *       phi(d2) dd + S + X e^{-rT}), eps = 2^-24, dd the conditioning of d1 (oracle).
  * The paper's CPU/GPU work split (25/75 on its laptop) is not built: there

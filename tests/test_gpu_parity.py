@@ -176,7 +176,7 @@ def test_tune_choice_is_valid_and_cached(tmp_path):
 
 
 def test_run_host_pipeline():
-    h, w, K = 2500, 16384, 5                                 # 3 row bands of 1024 rows
+    h, w, K = 2500, 16384, 5                                 # 10 row bands of 256 rows (16 MB chunks)
     img = synth.uniform_image(h, w, seed=21)
     k = synth.binomial_kernel(K)
     src = torch.from_numpy(img).pin_memory()
