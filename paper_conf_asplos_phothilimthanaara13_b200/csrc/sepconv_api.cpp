@@ -5,6 +5,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <array>
 #include <cmath>
 #include <cstdio>
 #include <cstdlib>
@@ -193,19 +194,18 @@ struct Sched {
     int grid, parts, win_rows, extra;
 };
 
-static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K) {
-    const long long slots = static_cast<long long>(di.sms) * occ;
+static Sched schedule_uncached(long long slots, int nimg, int nstrips, int rows, int K, bool no_win, bool force_win) {
     const long long strips = static_cast<long long>(nimg) * nstrips;
-    const long long min_rows = std::max(8, 4 * (K - 1));
+    // segments may be short: the score below already charges each one its K-1 warm-up rows,
+    // and on small images (2048^2: 2 CTA strips) a floor of 4(K-1) rows left 86 of 148 SMs
+    // idle at K=17 -- fill beats warm-up there
+    const long long min_rows = 8;
     const long long max_parts = std::max<long long>(1, rows / min_rows);
     const double o = (K - 1) + 16.0;                           // warm-up + pipeline fill, rows
     double best = -1.0;
     long long best_p = 0, best_g = 0;
     Sched win{0, 0, 0, 0};
     double win_score = -1.0;
-    const char *mode = std::getenv("SEPCONV_SCHED");          // read per launch: tests flip it
-    const bool no_win = mode && std::strcmp(mode, "nowin") == 0;
-    const bool force_win = mode && std::strcmp(mode, "win") == 0;
     if (!no_win && strips < slots && slots % strips != 0) {
         const long long q = slots / strips, e = slots - q * strips;
         const long long m = (strips + e - 1) / e;
@@ -249,6 +249,28 @@ static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int 
     if (win_score > 0 && (force_win || (win_score > best && win_score > contig_score))) return win;
     if (best_p > 0 && best >= contig_score) return Sched{static_cast<int>(best_g), static_cast<int>(best_p), 0, 0};
     return Sched{static_cast<int>(std::max<long long>(g_contig, 1)), 0, 0, 0};
+}
+
+// The search above walks up to 2 x 4096 part counts (~10 us of host time at 16384^2): memoised
+// per (slots, images, strips, rows, K, mode), so a steady-state sepconv_run only looks it up.
+static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K) {
+    const char *mode = std::getenv("SEPCONV_SCHED");          // read per launch: tests flip it
+    const bool no_win = mode && std::strcmp(mode, "nowin") == 0;
+    const bool force_win = mode && std::strcmp(mode, "win") == 0;
+    const long long slots = static_cast<long long>(di.sms) * occ;
+    static std::mutex mu;
+    static std::map<std::array<long long, 6>, Sched> memo;
+    const std::array<long long, 6> key{slots, nimg, nstrips, rows, K, no_win ? 1 : (force_win ? 2 : 0)};
+    {
+        std::lock_guard<std::mutex> lock(mu);
+        auto it = memo.find(key);
+        if (it != memo.end()) return it->second;
+    }
+    const Sched sc = schedule_uncached(slots, nimg, nstrips, rows, K, no_win, force_win);
+    std::lock_guard<std::mutex> lock(mu);
+    if (memo.size() > 4096) memo.clear();
+    memo[key] = sc;
+    return sc;
 }
 
 // One streaming pass (ROWS, COLS or SEP) over geometry g.
