@@ -213,23 +213,30 @@ __device__ __forceinline__ void bar_wait(uint64_t *bar, uint32_t parity) {
     } while (!done);
 }
 
-// relax4 with the parity a compile-time constant (the 6-step unroll fixes it)
+// relax4 with the parity a compile-time constant (the 6-step unroll fixes it).  All four
+// cells are evaluated and the frame / out-of-range cells then select their old value: a
+// select per cell instead of a predicated FADD/FFMA chain plus a move (same bits: the
+// arithmetic of every written cell is unchanged, P6)
 template <int S>
 __device__ __forceinline__ float4 relax4s(const float4 &u, const float4 &N, const float4 &Sv, const float4 &C,
                                           float left, float right, const float4 &b, unsigned msk, float w4,
                                           float om1) {
     float4 o;
     if constexpr (S == 0) {
-        o.x = (msk & 1u) ? relax1(N.x, Sv.x, left, C.x, b.x, u.x, w4, om1) : u.x;
-        o.y = (msk & 2u) ? relax1(N.y, Sv.y, C.x, C.y, b.y, u.y, w4, om1) : u.y;
-        o.z = (msk & 4u) ? relax1(N.z, Sv.z, C.y, C.z, b.z, u.z, w4, om1) : u.z;
-        o.w = (msk & 8u) ? relax1(N.w, Sv.w, C.z, C.w, b.w, u.w, w4, om1) : u.w;
+        o.x = relax1(N.x, Sv.x, left, C.x, b.x, u.x, w4, om1);
+        o.y = relax1(N.y, Sv.y, C.x, C.y, b.y, u.y, w4, om1);
+        o.z = relax1(N.z, Sv.z, C.y, C.z, b.z, u.z, w4, om1);
+        o.w = relax1(N.w, Sv.w, C.z, C.w, b.w, u.w, w4, om1);
     } else {
-        o.x = (msk & 1u) ? relax1(N.x, Sv.x, C.x, C.y, b.x, u.x, w4, om1) : u.x;
-        o.y = (msk & 2u) ? relax1(N.y, Sv.y, C.y, C.z, b.y, u.y, w4, om1) : u.y;
-        o.z = (msk & 4u) ? relax1(N.z, Sv.z, C.z, C.w, b.z, u.z, w4, om1) : u.z;
-        o.w = (msk & 8u) ? relax1(N.w, Sv.w, C.w, right, b.w, u.w, w4, om1) : u.w;
+        o.x = relax1(N.x, Sv.x, C.x, C.y, b.x, u.x, w4, om1);
+        o.y = relax1(N.y, Sv.y, C.y, C.z, b.y, u.y, w4, om1);
+        o.z = relax1(N.z, Sv.z, C.z, C.w, b.z, u.z, w4, om1);
+        o.w = relax1(N.w, Sv.w, C.w, right, b.w, u.w, w4, om1);
     }
+    o.x = (msk & 1u) ? o.x : u.x;
+    o.y = (msk & 2u) ? o.y : u.y;
+    o.z = (msk & 4u) ? o.z : u.z;
+    o.w = (msk & 8u) ? o.w : u.w;
     return o;
 }
 
