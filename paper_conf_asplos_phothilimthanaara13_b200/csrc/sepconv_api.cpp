@@ -56,6 +56,21 @@ static EncodeTiledFn encode_fn() {
     return fn;
 }
 
+sepconv_status_t encode_tmap_f32_3d(CUtensorMap *map, const float *base, const uint64_t dims[3],
+                                    const uint64_t strides_bytes[2], const uint32_t box[3]) {
+    EncodeTiledFn enc = encode_fn();
+    if (!enc) return fail(SEPCONV_E_CUDA, "cuTensorMapEncodeTiled unavailable from the driver");
+    cuuint64_t d[3] = {dims[0], dims[1], dims[2]};
+    cuuint64_t st[2] = {strides_bytes[0], strides_bytes[1]};
+    cuuint32_t bx[3] = {box[0], box[1], box[2]};
+    cuuint32_t estr[3] = {1, 1, 1};
+    CUresult r = enc(map, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<float *>(base), d, st, bx, estr,
+                     CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (r != CUDA_SUCCESS) return fail(SEPCONV_E_CUDA, "cuTensorMapEncodeTiled failed (CUresult %d)", (int)r);
+    return SEPCONV_OK;
+}
+
 static sepconv_status_t query_device(int device, DeviceInfo *out) {
     int count = 0;
     cudaError_t e = cudaGetDeviceCount(&count);

@@ -18,6 +18,10 @@ namespace sepconv {
 // ---- errors --------------------------------------------------------------------------
 sepconv_status_t fail(sepconv_status_t st, const char *fmt, ...);
 sepconv_status_t cuda_fail(cudaError_t e, const char *what);
+// cuTensorMapEncodeTiled for a float32 3-D tensor (dims innermost first, byte strides of dims 1
+// and 2), no swizzle, zero fill out of bounds; the driver entry point is resolved once
+sepconv_status_t encode_tmap_f32_3d(CUtensorMap *map, const float *base, const uint64_t dims[3],
+                                    const uint64_t strides_bytes[2], const uint32_t box[3]);
 extern std::atomic<uint64_t> g_launches;
 
 #define SC_CUDA(call)                                              \

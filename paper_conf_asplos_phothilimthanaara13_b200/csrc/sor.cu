@@ -39,7 +39,9 @@ constexpr int kMaxDepth = 8;
 constexpr int kWaveWarps = 4;            // warps per CTA of the wave kernel
 constexpr int kThreads = 256;            // split / merge / half kernels
 
-struct SorParams {
+struct alignas(64) SorParams {
+    CUtensorMap tmap;                    // WAVE: 3-D map {ldh, n, 6} over the plan's six split buffers
+    int zu;                              // WAVE: buffer index (0 or 2) of the pair the pass reads
     const float *ur, *ub;                // iterate read by the pass (split buffers)
     float *ur_out, *ub_out;              // iterate written (HALF: the same buffers)
     const float *br, *bb;                // right-hand side, split
@@ -188,11 +190,16 @@ __device__ __forceinline__ uint32_t smem_addr(const void *p) {
     return static_cast<uint32_t>(__cvta_generic_to_shared(p));
 }
 
-__device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t bytes, uint64_t *bar) {
-    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
-                     smem_addr(dst)),
-                 "l"(src), "r"(bytes), "r"(smem_addr(bar))
-                 : "memory");
+// one TMA box {128 split columns, 1 row, 2 buffers}: the red and the black row of one
+// buffer pair, 1 KB, columns outside [0, ldh) and rows outside [0, n) zero-filled (those cells
+// are never written and only feed cells that are not)
+__device__ __forceinline__ void tma_row_pair(void *dst, const CUtensorMap *map, uint64_t *bar, int col, int row,
+                                             int z) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
+        "[%0], [%1, {%3, %4, %5}], [%2];" ::"r"(smem_addr(dst)),
+        "l"(reinterpret_cast<uint64_t>(map)), "r"(smem_addr(bar)), "r"(col), "r"(row), "r"(z)
+        : "memory");
 }
 
 __device__ __forceinline__ void bar_expect(uint64_t *bar, uint32_t bytes) {
@@ -240,23 +247,23 @@ __device__ __forceinline__ float4 relax4s(const float4 &u, const float4 &N, cons
     return o;
 }
 
-// Rows reach shared memory through a per-warp ring filled by 1-D bulk copies (lane 0,
-// PF rows ahead, one mbarrier per u-ring slot covering the row's four copies: u red, u
-// black, b red, b black -- 512 B each); the b ring is deeper because the deepest level
+// Rows reach shared memory through a per-warp ring filled by TMA (lane 0, PF rows ahead, one
+// mbarrier per u-ring slot covering the row's two boxes: u red + black, b red + black --
+// 1 KB each, one 3-D tensor map over the six split buffers); the b ring is deeper because the deepest level
 // still needs b of row r - 2T.  The step loop is unrolled 6 ways from a row that is a
 // multiple of 6, so the 3-row window slots (row % 3) and the row parities (which
 // neighbour column a cell needs, hence which single shuffle) are compile-time constants.
 // (Measured alternatives: waiting once per 6-row block lets steps
 // overlap but needs 36 KB of ring per warp -- 4 warps/SM -- and ran 20% slower.)
 template <int T>
-__global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorParams p) {
+__global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_constant__ SorParams p) {
     using WV = Wave<T>;
     constexpr int HL = WV::HL, WOUT = WV::WOUT, PF = WV::PF, RDU = WV::RDU, RDB = WV::RDB;
     extern __shared__ __align__(128) float wsmem[];
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     float *ring = wsmem + warp * WV::WARP_FLOATS;
-    float *ringU0 = ring, *ringU1 = ring + 128 * RDU;                     // u red, u black
-    float *ringB0 = ring + 256 * RDU, *ringB1 = ring + 256 * RDU + 128 * RDB;   // b red, b black
+    float *ringU = ring;                                                 // [RDU][red, black][128] of u
+    float *ringB = ring + 256 * RDU;                                     // [RDB][red, black][128] of b
     uint64_t *bars = reinterpret_cast<uint64_t *>(wsmem + kWaveWarps * WV::WARP_FLOATS) + warp * RDU;
     if (lane == 0) {
 #pragma unroll
@@ -287,10 +294,6 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
         const int k0 = kbase + 4 * lane;
         const bool writer = lane >= HL && lane < 32 - HL && k0 < ldh;
         const unsigned m0 = col_mask(k0, 0, p.m, ldh), m1 = col_mask(k0, 1, p.m, ldh);
-        // the in-range part of the strip's 128 columns (bulk copies stay inside the rows)
-        const int g0 = max(kbase, 0), g1 = min(kbase + 128, static_cast<int>(ldh));
-        const uint32_t cbytes = static_cast<uint32_t>(g1 - g0) * 4u;
-        const int soff = g0 - kbase;
         int r0 = max(0, q0 - 2 * T);
         r0 -= r0 % 6;
         const int nsteps = ((q1 - 1 + 2 * T) - r0) / 6 * 6 + 6;           // whole 6-step blocks
@@ -300,17 +303,9 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
         auto issue = [&](int j) {                                        // step j = row r0 + j
             const uint32_t cc = c0 + j;
             uint64_t *bar = &bars[cc % RDU];
-            const int row = r0 + j;
-            if (row < n) {
-                const long long go = static_cast<long long>(row) * ldh + g0;
-                bar_expect(bar, 4 * cbytes);
-                bulk_g2s(ringU0 + (cc % RDU) * 128 + soff, p.ur + go, cbytes, bar);
-                bulk_g2s(ringU1 + (cc % RDU) * 128 + soff, p.ub + go, cbytes, bar);
-                bulk_g2s(ringB0 + (cc % RDB) * 128 + soff, p.br + go, cbytes, bar);
-                bulk_g2s(ringB1 + (cc % RDB) * 128 + soff, p.bb + go, cbytes, bar);
-            } else {
-                bar_expect(bar, 0);                                      // past the grid: complete the phase
-            }
+            bar_expect(bar, 2 * 1024);                                   // full boxes, OOB included
+            tma_row_pair(ringU + (cc % RDU) * 256, &p.tmap, bar, kbase, r0 + j, p.zu);
+            tma_row_pair(ringB + (cc % RDB) * 256, &p.tmap, bar, kbase, r0 + j, 4);
         };
         __syncwarp();                                                    // every lane is past the last segment
         if (lane == 0) {
@@ -340,8 +335,8 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
                 }
                 bar_wait(&bars[cc % RDU], (cc / RDU) & 1);
                 __syncwarp();
-                R[0][u % 3] = *reinterpret_cast<const float4 *>(ringU0 + (cc % RDU) * 128 + 4 * lane);
-                B[0][u % 3] = *reinterpret_cast<const float4 *>(ringU1 + (cc % RDU) * 128 + 4 * lane);
+                R[0][u % 3] = *reinterpret_cast<const float4 *>(ringU + (cc % RDU) * 256 + 4 * lane);
+                B[0][u % 3] = *reinterpret_cast<const float4 *>(ringU + (cc % RDU) * 256 + 128 + 4 * lane);
 #pragma unroll
                 for (int t = 1; t <= T; ++t) {
                     {   // red_t at rho = r - 2t + 1 (parity of u + 1)
@@ -349,7 +344,7 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
                         const float4 C = B[t - 1][sc];
                         const bool row_in = static_cast<unsigned>(r - 2 * t) < nm2;   // rho - 1 < n - 2
                         const float4 b = *reinterpret_cast<const float4 *>(
-                            ringB0 + ((cc - (2 * t - 1)) % RDB) * 128 + 4 * lane);
+                            ringB + ((cc - (2 * t - 1)) % RDB) * 256 + 4 * lane);
                         if ((u + 1) % 2 == 0) {                             // rho even: red at even columns
                             const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
                             R[t][sc] = relax4s<0>(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, left, 0.f, b,
@@ -365,7 +360,7 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const SorPara
                         const float4 C = R[t][sc];
                         const bool row_in = static_cast<unsigned>(r - 2 * t - 1) < nm2;
                         const float4 b = *reinterpret_cast<const float4 *>(
-                            ringB1 + ((cc - 2 * t) % RDB) * 128 + 4 * lane);
+                            ringB + ((cc - 2 * t) % RDB) * 256 + 128 + 4 * lane);
                         if ((u + 1) % 2 == 0) {
                             const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
                             B[t][sc] = relax4s<0>(B[t - 1][sc], R[t][sm], R[t][sp], C, left, 0.f, b,
@@ -417,6 +412,7 @@ struct sor_plan_s {
     int variant = -1, depth = 0;     // tuned (variant < 0: untuned)
     int forced_depth = 0;
     int wave_occ[sor::kMaxDepth + 1] = {};
+    CUtensorMap tmap;                // {ldh, n, 6} over buf (the wave kernel's TMA source)
     // row bands (sor_comm_init): this plan holds rows [row0 - h_top, row1 + h_bot) of the grid
     bool band = false, band_external = false;
     void *comm = nullptr;
@@ -475,6 +471,8 @@ sepconv_status_t wave_pass(sor_plan_t plan, float omega, int T, cudaStream_t st)
     p.ub = plan->u[src][1];
     p.ur_out = plan->u[dst][0];
     p.ub_out = plan->u[dst][1];
+    p.tmap = plan->tmap;
+    p.zu = 2 * src;
     int &occ = plan->wave_occ[T];
     if (occ == 0) {
         static const void *funcs[sor::kMaxDepth + 1] = {
@@ -562,6 +560,17 @@ sepconv_status_t sor_plan(int64_t n, int64_t m, sor_plan_t *out) {
     p->u[1][1] = p->buf + 3 * one;
     p->b[0] = p->buf + 4 * one;
     p->b[1] = p->buf + 5 * one;
+    {
+        const uint64_t dims[3] = {static_cast<uint64_t>(p->ldh), static_cast<uint64_t>(n), 6};
+        const uint64_t strides[2] = {static_cast<uint64_t>(p->ldh) * 4, one * 4};
+        const uint32_t box[3] = {128, 1, 2};
+        sepconv_status_t st = sepconv::encode_tmap_f32_3d(&p->tmap, p->buf, dims, strides, box);
+        if (st != SEPCONV_OK) {
+            cudaFree(p->buf);
+            delete p;
+            return st;
+        }
+    }
     e = cudaMemset(p->buf, 0, 6 * one * sizeof(float));
     if (e != cudaSuccess) {
         cudaFree(p->buf);
