@@ -17,8 +17,9 @@
 //   sor_wave_kernel<T>                  T iterations in one pass (SOR_WAVE): each warp
 //       owns a strip of 4*(32-2*HL) split columns (HL halo lanes per side, HL =
 //       ceil(2T/4): the dependency cone widens by one split column per half-sweep) and
-//       walks down its rows.  Rows arrive in a per-warp shared-memory ring by 1-D bulk
-//       copies (cp.async.bulk + mbarrier) PF rows ahead.  At step r the warp takes row
+//       walks down its rows.  Rows arrive in a per-warp shared-memory ring by 3-D TMA
+//       (cp.async.bulk.tensor + mbarrier; one box = the red and black row of a buffer
+//       pair) PF rows ahead.  At step r the warp takes row
 //       r (level 0) and computes red_t(r-2t+1), black_t(r-2t) for t = 1..T from 3-row
 //       register windows of the previous level, so u and b are read once and u written
 //       once per T iterations (12 B per cell per pass), out of place into the plan's
