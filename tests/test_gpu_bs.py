@@ -100,3 +100,26 @@ def test_errors():
         bs.price(a, a, a, R, V, a, out)
     assert ei.value.code == "E_ALIAS"
     bs.price(a, a, a, R, V, out, torch.empty(16, device="cuda"), n=0)   # no-op
+
+
+@pytest.mark.parametrize("v", [0.01, 0.3, 2.0])
+def test_extreme_moneyness_expiry_and_volatility(v):
+    """The normal-CDF tails (reading B5: the Chebyshev erfc and N / 1 - N from one tail value)
+    and the SFU transcendentals (B3) over a grid far outside the benchmark ranges: S/X from
+    1e-2 to 1e2 (|d| up to ~450 at v = 0.01, deep in both tails), T from 1e-3 to 30 years,
+    at-the-money-forward points where d1 ~ 0."""
+    ratio = np.geomspace(1e-2, 1e2, 257)
+    years = np.geomspace(1e-3, 30.0, 33)
+    rr, tt = np.meshgrid(ratio, years)
+    x = np.full(rr.size, 50.0, np.float32)
+    s = (x * rr.reshape(-1)).astype(np.float32)
+    t = tt.reshape(-1).astype(np.float32)
+    # at-the-money-forward: S = X exp(-(r + v^2/2) T) makes d1 = 0 up to rounding
+    atm_t = np.geomspace(1e-3, 30.0, 64).astype(np.float32)
+    atm_s = (50.0 * np.exp(-(R + 0.5 * v * v) * atm_t.astype(np.float64))).astype(np.float32)
+    s = np.concatenate([s, atm_s])
+    x = np.concatenate([x, np.full(atm_s.size, 50.0, np.float32)])
+    t = np.concatenate([t, atm_t])
+    c, p = gpu_price(s, x, t, R, v)
+    check(s, x, t, c, p, R, v)
+    assert np.all(c >= -1e-6 * (s + x)) and np.all(p >= -1e-6 * (s + x))      # no-arbitrage lower bounds
