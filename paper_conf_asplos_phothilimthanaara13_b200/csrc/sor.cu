@@ -321,7 +321,17 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_
             for (int z = 0; z < 3; ++z) R[t][z] = B[t][z] = make_float4(0.f, 0.f, 0.f, 0.f);
 
 #pragma unroll 1
+        const float *ringBl = ringB + 4 * lane;                           // this lane's column of the b ring
         for (int jb = 0; jb < nsteps; jb += 6) {
+            // b-ring slot of step jb; slots of the unrolled steps and levels are compile-time
+            // offsets from it with one conditional wrap (no division by RDB per load)
+            const int hb = static_cast<int>((c0 + jb) % RDB);
+            auto bslot = [&](int off) -> const float * {                 // slot of counter c0 + jb + off
+                int v = hb + off;
+                if (off < 0) v += (hb < -off) ? RDB : 0;
+                if (off > 0) v -= (hb >= RDB - off) ? RDB : 0;
+                return ringBl + v * 256;
+            };
 #pragma unroll
             for (int u = 0; u < 6; ++u) {
                 const int j = jb + u;
@@ -345,7 +355,7 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_
                         const float4 C = B[t - 1][sc];
                         const bool row_in = static_cast<unsigned>(r - 2 * t) < nm2;   // rho - 1 < n - 2
                         const float4 b = *reinterpret_cast<const float4 *>(
-                            ringB + ((cc - (2 * t - 1)) % RDB) * 256 + 4 * lane);
+                            bslot(u - (2 * t - 1)));
                         if ((u + 1) % 2 == 0) {                             // rho even: red at even columns
                             const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
                             R[t][sc] = relax4s<0>(R[t - 1][sc], B[t - 1][sm], B[t - 1][sp], C, left, 0.f, b,
@@ -361,7 +371,7 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_
                         const float4 C = R[t][sc];
                         const bool row_in = static_cast<unsigned>(r - 2 * t - 1) < nm2;
                         const float4 b = *reinterpret_cast<const float4 *>(
-                            ringB + ((cc - 2 * t) % RDB) * 256 + 128 + 4 * lane);
+                            bslot(u - 2 * t) + 128);
                         if ((u + 1) % 2 == 0) {
                             const float left = __shfl_up_sync(0xffffffffu, C.w, 1);
                             B[t][sc] = relax4s<0>(B[t - 1][sc], R[t][sm], R[t][sp], C, left, 0.f, b,
