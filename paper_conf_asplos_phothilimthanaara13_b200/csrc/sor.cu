@@ -320,8 +320,8 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_
 #pragma unroll
             for (int z = 0; z < 3; ++z) R[t][z] = B[t][z] = make_float4(0.f, 0.f, 0.f, 0.f);
 
-#pragma unroll 1
         const float *ringBl = ringB + 4 * lane;                           // this lane's column of the b ring
+#pragma unroll 1
         for (int jb = 0; jb < nsteps; jb += 6) {
             // b-ring slot of step jb; slots of the unrolled steps and levels are compile-time
             // offsets from it with one conditional wrap (no division by RDB per load)
