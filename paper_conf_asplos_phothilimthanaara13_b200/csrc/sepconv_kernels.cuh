@@ -486,8 +486,10 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             }
             if constexpr (TMA) {
                 if constexpr (LOCK) {
-                    // CTA lockstep: the active warps of this strip finish the stage together
-                    asm volatile("bar.sync 1, %0;" ::"r"(lock_threads) : "memory");
+                    // CTA lockstep: the active warps of this strip finish the stage together.
+                    // Non-.aligned barrier: the edge warp of a strip runs the other copy of this
+                    // loop (scalar stores), i.e. a different barrier instruction with the same id
+                    asm volatile("barrier.sync 1, %0;" ::"r"(lock_threads) : "memory");
                 } else {
                     __syncwarp();
                 }

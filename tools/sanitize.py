@@ -10,7 +10,8 @@ from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc  # noqa: E4
 from paper_conf_asplos_phothilimthanaara13_b200 import synth  # noqa: E402
 
 Ks = [int(x) for x in sys.argv[1].split(",")] if len(sys.argv) > 1 else [3, 17]
-for (h, w) in ((40, 1100), (67, 131)):
+# (1200, 700) and (300, 4200): many short segments, several per CTA (the schedule allows 8-row segments)
+for (h, w) in ((40, 1100), (67, 131), (1200, 700), (300, 4200)):
     img = torch.from_numpy(synth.uniform_image(h, w, seed=1)).cuda()
     for K in Ks:
         if K > min(h, w):
