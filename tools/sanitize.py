@@ -22,3 +22,23 @@ for (h, w) in ((40, 1100), (67, 131), (1200, 700), (300, 4200)):
             p.run_choice(img, synth.binomial_kernel(K), out, c)
             torch.cuda.synchronize()
             print("ok", h, w, K, c.name, flush=True)
+
+# the host pipeline (banded copy-in / kernel / copy-out) and row bands in external-halo mode
+h, w, K = 700, 2100, 5
+img = synth.uniform_image(h, w, seed=2)
+src = torch.from_numpy(img).pin_memory()
+dst = torch.empty((h - K + 1, w - K + 1)).pin_memory()
+p = sc.Plan(h, w, K)
+for v in ("separable", "2d"):
+    p.run_host(src, synth.binomial_kernel(K), dst, v)
+    print("ok run_host", v, flush=True)
+dev = torch.from_numpy(img).cuda()
+for g in range(2):
+    r0, rows, owned, alloc = sc.band(h, K, 2, g)
+    band = dev[r0:r0 + alloc].contiguous()
+    q = sc.Plan(alloc, w, K)
+    q.comm_init(None, 2, g)
+    out = torch.empty((rows, w - K + 1), device="cuda")
+    q.run_band(band, synth.binomial_kernel(K), out, "auto")
+    torch.cuda.synchronize()
+    print("ok run_band", g, flush=True)
