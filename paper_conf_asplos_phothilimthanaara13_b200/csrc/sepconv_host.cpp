@@ -87,11 +87,19 @@ extern "C" sepconv_status_t sepconv_run_host(sepconv_plan_t plan, const float *i
             const int slot = static_cast<int>(i & 1);
             const int64_t rr = std::min<int64_t>(R, plan->ho - r0);
             const int64_t rin = rr + K - 1;
-            // copy-in: input rows [r0, r0 + rr + K - 1) of image n
+            // copy-in: input rows [r0, r0 + rr + K - 1) of image n.  The first K-1 of
+            // them are the previous band's last K-1 rows, already on the device in the other slot
+            // (its copy-in precedes this one on sh): a device-to-device copy, so PCIe carries every
+            // input row once (the H2D direction bounds the pipeline)
             if (i >= 2) SC_CUDA(cudaStreamWaitEvent(sh, ev[1][slot], 0));
-            SC_CUDA(cudaMemcpy2DAsync(plan->hin[slot], plan->ld_in * 4,
-                                      in_host + (n * plan->h + r0) * plan->ld_in, plan->ld_in * 4, plan->w * 4,
-                                      rin, cudaMemcpyHostToDevice, sh));
+            const int64_t carry = (r0 > 0) ? K - 1 : 0;
+            if (carry > 0)
+                SC_CUDA(cudaMemcpy2DAsync(plan->hin[slot], plan->ld_in * 4,
+                                          plan->hin[slot ^ 1] + R * plan->ld_in, plan->ld_in * 4, plan->w * 4,
+                                          carry, cudaMemcpyDeviceToDevice, sh));
+            SC_CUDA(cudaMemcpy2DAsync(plan->hin[slot] + carry * plan->ld_in, plan->ld_in * 4,
+                                      in_host + (n * plan->h + r0 + carry) * plan->ld_in, plan->ld_in * 4,
+                                      plan->w * 4, rin - carry, cudaMemcpyHostToDevice, sh));
             SC_CUDA(cudaEventRecord(ev[0][slot], sh));
             // execute
             SC_CUDA(cudaStreamWaitEvent(sc, ev[0][slot], 0));
