@@ -194,11 +194,26 @@ struct OutCursor {
             : "memory");
         ptr += ld;
     }
-    // MODE 2: 16-byte rows, 1: 8-byte rows, 0: ragged edge / 4-byte rows
+    // 8-byte rows without shuffles: two predicated 8-byte stores per lane (each 32-byte sector
+    // is written in two halves by the two instructions); fewer live registers than store_fast
+    __device__ __forceinline__ void store_v2x2(const float (&v)[V], bool ok) {
+        const unsigned q = ok;
+        asm volatile(
+            "{\n\t.reg .pred q8;\n\t"
+            "setp.ne.u32 q8, %5, 0;\n\t"
+            "@q8 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
+            "@q8 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(q)
+            : "memory");
+        ptr += ld;
+    }
+    // MODE 2: 16-byte rows, 1: 8-byte rows (shuffled into 16-byte chunks), 3: 8-byte rows as
+    // two 8-byte stores, 0: ragged edge / 4-byte rows
     template <int MODE>
     __device__ __forceinline__ void put(const float (&v)[V], bool ok, int lane) {
         if constexpr (MODE == 2) store_fast16(v, ok);
         else if constexpr (MODE == 1) store_fast(v, ok, lane);
+        else if constexpr (MODE == 3) store_v2x2(v, ok);
         else store_scalar(v, ok);
     }
     // write v to the cursor row if ok, then move to the next row
@@ -503,7 +518,10 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         };
         // SM (a template parameter) is the store path of warps wholly inside the image; the
         // host instantiates SM = 2 when every row start is 16-byte aligned, else SM = 1
-        if (wcol + kWarpCols <= p.out_cols && p.store8 >= SM) run_chunks(std::integral_constant<int, SM>{});
+        // (16-warp configurations take the 8-byte rows as two 8-byte stores: the shuffled form
+        // spills at their 128-register budget)
+        constexpr int SMF = (SM == 1 && NW >= 16) ? 3 : SM;
+        if (wcol + kWarpCols <= p.out_cols && p.store8 >= SM) run_chunks(std::integral_constant<int, SMF>{});
         else run_chunks(std::integral_constant<int, 0>{});
     }
 }
