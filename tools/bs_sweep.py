@@ -1,5 +1,7 @@
-"""Time bs_price on 2^28 device-resident options (median of 20, CUDA events);
-select the exploration variant.  python tools/bs_sweep.py"""
+"""Time bs_price on 2^28 device-resident options (median of 20, CUDA events).
+    python tools/bs_sweep.py
+(profiles/r01_bs_sweep.txt was taken with temporary BS_U / BS_CPS environment switches for the
+unroll and the grid size; the kernel now hard-codes the winner: U = 2, 4 CTAs per SM.)"""
 import os, sys, statistics
 sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import torch
