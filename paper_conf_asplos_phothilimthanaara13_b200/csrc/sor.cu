@@ -507,13 +507,17 @@ sepconv_status_t wave_pass(sor_plan_t plan, float omega, int T, cudaStream_t st)
         if (e != cudaSuccess) return cuda_fail(e, "sor wave occupancy");
         occ = std::max(occ, 1);
     }
-    // items = strips x row segments, about one per resident warp (each segment pays 4T
-    // warm-up/drain steps: keep segments >= 16T rows)
+    // items = strips x row segments, about one per resident warp.  Each segment pays ~4T
+    // warm-up/drain steps, but idle warps cost more: on the paper's 2048^2 a floor of 16T rows
+    // per segment left three quarters of the warps idle (372 G vs 565 G cell-it/s at T=3,
+    // profiles/r01_sor_perf.txt), so segments only keep >= 2T rows.  Segment rows are a multiple
+    // of the 6-step unroll, so every segment starts on a block boundary and no steps are wasted
+    // aligning its first block.
     p.nstrips = static_cast<int>((plan->ldh + sor::kWout[T] - 1) / sor::kWout[T]);
     const long long warps = static_cast<long long>(plan->sms) * occ * sor::kWaveWarps;
     long long nsegs = std::max<long long>(1, warps / p.nstrips);
-    nsegs = std::min<long long>(nsegs, std::max<long long>(1, plan->n / (16 * T)));
-    p.seg_rows = static_cast<int>((plan->n + nsegs - 1) / nsegs);
+    nsegs = std::min<long long>(nsegs, std::max<long long>(1, plan->n / (2 * T)));
+    p.seg_rows = static_cast<int>(((plan->n + nsegs - 1) / nsegs + 5) / 6 * 6);
     nsegs = (plan->n + p.seg_rows - 1) / p.seg_rows;
     p.items = nsegs * p.nstrips;
     const long long blocks = (p.items + sor::kWaveWarps - 1) / sor::kWaveWarps;
