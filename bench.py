@@ -184,7 +184,9 @@ def run_reference(args):
     W = args.size if args.workload == "image" else 4096
     H = W
     seed = synth.BENCH_SEED_BASE + (3 if args.workload == "image" else 4)
-    per_step_s = max(2.0, 60.0 / max(1, args.steps + args.warmup))
+    # each step a bounded sample: about a minute for the whole --steps/--warmup run, at most
+    # --cpu-seconds per step (tests pass a small value)
+    per_step_s = max(0.2, min(args.cpu_seconds, 60.0 / max(1, args.steps + args.warmup)))
     rows_cache = {}
 
     def img_rows(n):
@@ -201,8 +203,12 @@ def run_reference(args):
         vals.append(last["value"])
         times.append(last["seconds"])
     value = statistics.median(vals)
-    cfg = {"workload": "16384x16384 float32 image, widths 3..17 odd" if args.workload == "image"
-           else "64 x 4096x4096 float32, width 11", "widths": widths, "sample": last["sample"]}
+    # the same workload string and keys as the CUDA arm's line (the oracle times a sample of it)
+    cfg = {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
+                        if args.workload == "image" else f"64 x {H}x{W} float32 images, width 11"),
+           "image": [H, W], "images": 1 if args.workload == "image" else 64, "widths": widths,
+           "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed, "sample": last["sample"],
+           "parallelism": "host cores (oracle)"}
     emit({"impl": "reference", "metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world,
           "steps": args.steps, "warmup": args.warmup, "ms_per_step": statistics.median(times) * 1e3,
           "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
