@@ -52,7 +52,9 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
         emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Moptions/s", "n_gpus": world,
               "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "weak",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-              "config": {"workload": "Black-Scholes (oracle sample)", "sample": last["sample"]},
+              "config": {"workload": (f"Black-Scholes, {args.options} float32 options per GPU "
+                                      f"(r={synth.BS_RATE}, v={synth.BS_VOL})"),
+                         "options": args.options, "sample": last["sample"], "parallelism": "host core (oracle)"},
               "cpu_baseline": {"value": v, "unit": "Moptions/s", "cores": 1, "kind": "oracle", "sample": last["sample"]},
               "e2e": {"value": v, "unit": "Moptions/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}})
         return 0

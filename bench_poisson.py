@@ -52,9 +52,12 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
                 vals.append(last["value"])
         v = statistics.median(vals)
         emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Mcell-it/s", "n_gpus": world,
-              "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "weak",
+              "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-              "config": {"workload": "Poisson2D red-black SOR (oracle sample)", "sample": last["sample"]},
+              "config": {"workload": (f"Poisson2D red-black SOR, {args.size}x{args.size} float32 grid, "
+                                      f"{args.sor_iters} iterations per step"),
+                         "grid": [args.size, args.size], "iters_per_step": args.sor_iters,
+                         "sample": last["sample"], "parallelism": "host core (oracle)"},
               "cpu_baseline": {"value": v, "unit": "Mcell-it/s", "cores": 1, "kind": "oracle", "sample": last["sample"]},
               "e2e": {"value": v, "unit": "Mcell-it/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}})
         return 0
