@@ -407,6 +407,12 @@ def main():
                 "unit": "GB/s", "frac": achieved / peak_gbs, "traffic": traffic, "peak_source": peak_src,
                 "algorithmic_bytes_per_launch": dom_bytes / len(dom_k),
                 "frac_of_8tbs": achieved / NOMINAL_HBM_GBS}
+    if dom_bytes < 256e6:
+        # a pass moving this little is bound by launch latency, pipeline fill and the K-1 warm-up
+        # rows of short segments (~5 us fixed per pass, profiles/r01_small_latency.txt), not by HBM
+        roofline["note"] = ("latency-bound: the pass moves %.1f MB; a fixed ~5 us per pass (launch, first TMA "
+                            "round trip, store drain) dominates, so frac is not an HBM-efficiency figure"
+                            % (dom_bytes / len(dom_k) / 1e6))
 
     # ---- e2e: the public API with pinned HOST buffers, copies inside the timed region ----
     e2e = None
