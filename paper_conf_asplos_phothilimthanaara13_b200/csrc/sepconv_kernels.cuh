@@ -387,6 +387,13 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
 
     int n, s, q0, nrows;
     while (seg.next(n, s, q0, nrows)) {
+        if constexpr (TMA && LOCK) {
+            // the lockstep barrier's thread count depends on the strip: a warp must not reach
+            // the next segment's barriers while another still uses this one's (a CTA whose
+            // segments span a full strip and a narrow right-edge strip of a batch or of a
+            // window schedule would otherwise mix counts on barrier 1)
+            __syncthreads();
+        }
         const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
         if (wcol >= p.out_cols) continue;
         // warps of this strip that have columns (named-barrier thread count for LOCK)

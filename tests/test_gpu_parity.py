@@ -188,6 +188,44 @@ def test_run_host_pipeline():
         check(img, k, dst.numpy())
 
 
+def test_batch_with_narrow_edge_strip_every_fused_config():
+    """A batch whose images end in a one-warp CTA strip (16400 columns: 16 full 1024-column
+    strips + 8 columns) under the window schedule: CTAs take segments of different strips, so
+    the lockstep configurations must not mix barrier counts between segments (a hang/trap
+    before the per-segment CTA barrier).  Every fused TMA configuration, both store paths."""
+    n, h, w, K = 2, 700, 16400, 9       # 692 output rows: q = 4 windows + 12 CTAs x 3 short segments
+    imgs = np.stack([synth.uniform_image(h, w, seed=91, n=i) for i in range(n)])
+    k = synth.binomial_kernel(K)
+    outs = [run_gpu(imgs, k, c) for c in CANDS if c.algo == sc.SEPCONV_SEPARABLE and c.fused]
+    for o in outs[1:]:
+        assert np.array_equal(o, outs[0])
+    for i in range(n):
+        check(imgs[i], k, outs[0][i])
+
+
+def test_run_host_batch_and_pitch_equal_device_run():
+    """Host pipeline over a batch (bands restart at every image: no halo carry across images)
+    with pitched buffers: bitwise equal to the device-resident run of the same plan."""
+    n, h, w, K = 2, 700, 16400, 9                          # 16 MB bands of 255 rows: 3 per image
+    imgs = np.stack([synth.uniform_image(h, w, seed=77, n=i) for i in range(n)])
+    ld_in, ld_out = w + 12, w - K + 1 + 5
+    src = np.zeros((n, h, ld_in), np.float32)
+    src[:, :, :w] = imgs
+    src_t = torch.from_numpy(src).pin_memory()
+    dst_t = torch.full((n, h - K + 1, ld_out), float("nan")).pin_memory()
+    k = synth.random_kernel(K, seed=3, signed=True)
+    p = sc.Plan(h, w, K, n=n, ld_in=ld_in, ld_out=ld_out)
+    p.run_host(src_t, k, dst_t, "separable")
+    dev_out = torch.full((n, h - K + 1, ld_out), float("nan"), device="cuda")
+    p.run(src_t.cuda(), k, dev_out, "separable")
+    torch.cuda.synchronize()
+    got = dst_t.numpy()
+    assert np.array_equal(got[:, :, :w - K + 1], dev_out.cpu().numpy()[:, :, :w - K + 1])
+    assert np.all(np.isnan(got[:, :, w - K + 1:]))                 # pitch padding untouched
+    for i in range(n):
+        check(imgs[i], k, got[i, :, :w - K + 1])
+
+
 def test_errors():
     p = sc.Plan(64, 64, 3)
     buf = torch.zeros(64 * 64 * 2, device="cuda")
