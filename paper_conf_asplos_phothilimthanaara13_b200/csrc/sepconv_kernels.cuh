@@ -410,7 +410,9 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         oc.init(out_rows - (RING ? static_cast<long long>(K - 1) * p.ld_out : 0LL), p.ld_out, c, p.out_cols);
 
         if constexpr (TMA) {
+            __syncwarp();                                      // every lane is past the previous segment's reads
             if (lane == 0) {
+                fence_proxy_async_smem();                      // ... which precede these async-proxy writes
                 const int npro = nchunks < NS ? nchunks : NS;
                 for (int ch = 0; ch < npro; ++ch) {
                     const int st = (kc + ch) % NS;
@@ -597,7 +599,9 @@ __global__ void __launch_bounds__(NW * 32, 1) conv2d_kernel(const __grid_constan
         oc.init(out_rows, p.ld_out, c, p.out_cols);
 
         if constexpr (TMA) {
+            __syncwarp();                                      // every lane is past the previous segment's reads
             if (lane == 0) {
+                fence_proxy_async_smem();                      // ... which precede these async-proxy writes
                 const int npro = nchunks < NS ? nchunks : NS;
                 for (int ch = 0; ch < npro; ++ch) {
                     const int st = (kc0 + ch) % NS;
