@@ -67,3 +67,51 @@ def test_random_configuration(seed):
                 sep_ref = got.copy()
             else:
                 assert np.array_equal(got, sep_ref), f"{c.name} differs from the other separable candidates"
+
+
+@pytest.mark.parametrize("seed", range(24))
+def test_random_sor_configuration(seed):
+    """Poisson2D red-black SOR: random grids, wavefront depths and
+    iteration counts (segment splits, ragged strips, partial last passes) bitwise equal to the
+    fixed-order float32 oracle."""
+    from paper_conf_asplos_phothilimthanaara13_b200 import sor
+    rng = np.random.default_rng(0x50F + seed)
+    n = int(rng.integers(3, 420))
+    m = int(rng.choice([int(rng.integers(3, 300)), int(rng.integers(200, 3000))]))
+    depth = int(rng.integers(1, 9))
+    iters = int(rng.integers(1, 10))
+    omega = float(rng.choice([1.0, 1.5, 1.9]))
+    x, b = synth.poisson_problem(n, m, seed=seed, guess="uniform")
+    want = oracle.sor_rb_f32(x, b, omega, iters)
+    with sor.SorPlan(n, m) as sp:
+        for v, d in (("wave", depth), ("half", 0)):
+            sp.set_depth(d)
+            u = torch.full((n, m), float("nan"), device="cuda")
+            sp.solve(torch.from_numpy(x).cuda(), torch.from_numpy(b).cuda(), u, omega, iters, v)
+            torch.cuda.synchronize()
+            assert np.array_equal(u.cpu().numpy(), want), f"{v} depth {d}: {n}x{m}, {iters} iterations"
+
+
+@pytest.mark.parametrize("seed", range(16))
+def test_random_black_scholes_configuration(seed):
+    """Black-Scholes: random counts (vector body + ragged tail), pointer
+    offsets (scalar path), rates and volatilities, within the B4 bound of the double oracle."""
+    from paper_conf_asplos_phothilimthanaara13_b200 import bs
+    rng = np.random.default_rng(0xB5 + seed)
+    n = int(rng.choice([int(rng.integers(1, 64)), int(rng.integers(1000, 300000))]))
+    off = int(rng.integers(0, 4))
+    r = float(rng.uniform(-0.02, 0.1))
+    v = float(rng.uniform(0.02, 1.2))
+    s, x, t = synth.bs_options(n, seed=seed)
+    dev = [torch.empty(n + off, dtype=torch.float32, device="cuda") for _ in range(5)]
+    for d, a in zip(dev[:3], (s, x, t)):
+        d[off:] = torch.from_numpy(a)
+    dev[3].fill_(float("nan"))
+    dev[4].fill_(float("nan"))
+    bs.price(dev[0][off:], dev[1][off:], dev[2][off:], r, v, dev[3][off:], dev[4][off:], n=n)
+    torch.cuda.synchronize()
+    oc, op, scale = oracle.black_scholes(s, x, t, r, v, with_scale=True)
+    for got, want in ((dev[3][off:], oc), (dev[4][off:], op)):
+        g = got.cpu().numpy()
+        assert not np.any(np.isnan(g))
+        assert np.all(np.abs(g - want) <= 16 * 2.0 ** -24 * scale)
