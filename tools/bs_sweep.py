@@ -18,4 +18,4 @@ for it in range(25):
     a.record(); bs.price(s, x, t, synth.BS_RATE, synth.BS_VOL, c, p); b.record(); torch.cuda.synchronize()
     if it >= 5: ts.append(a.elapsed_time(b))
 m = statistics.median(ts)
-print(f"U={os.environ.get('BS_U','1')} CPS={os.environ.get('BS_CPS','8')}: {m*1e3:.1f} us  {n/m/1e6:.0f} G opt/s  {20*n/m/1e6:.0f} GB/s")
+print(f"bs_kernel_vec<2>, 4 CTAs/SM: {m*1e3:.1f} us  {n/m/1e6:.0f} G opt/s  {20*n/m/1e6:.0f} GB/s")
