@@ -477,6 +477,10 @@ def main():
         else:
             cpu = oracle_sample(lambda n: host_img[0][:n], W, widths, args.cpu_seconds, H=H)
         cpu = {k: v for k, v in cpu.items() if k not in ("seconds", "pixels")}
+        if args.workload == "image" and H <= 256:
+            # the small case also reports the single-thread oracle
+            one = oracle_sample(lambda n: host_img[:n], W, widths, min(args.cpu_seconds, 3.0), nthreads=1, H=H)
+            cpu["single_thread"] = {"value": one["value"], "unit": "Mpixels/s", "cores": 1, "sample": one["sample"]}
 
     if rank == 0:
         cfg = {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
