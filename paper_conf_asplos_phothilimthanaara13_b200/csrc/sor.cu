@@ -191,6 +191,27 @@ __device__ __forceinline__ uint32_t smem_addr(const void *p) {
     return static_cast<uint32_t>(__cvta_generic_to_shared(p));
 }
 
+// One step's refill issued by the whole (converged) warp: the operands are warp-uniform values
+// computed outside any lane-divergent branch, and one elected lane runs the fence, the
+// expect_tx and the two TMA boxes (u pair, b pair) under a predicate -- no `if (lane == 0)`
+// region whose operands ptxas would move into uniform registers lane by lane.
+__device__ __forceinline__ void refill_elected(bool go, uint32_t bar, uint32_t dst_u, uint32_t dst_b,
+                                               const CUtensorMap *map, int col, int row, int zu) {
+    asm volatile(
+        "{\n\t.reg .pred e, g, q;\n\t"
+        "elect.sync _|e, 0xffffffff;\n\t"
+        "setp.ne.u32 g, %0, 0;\n\t"
+        "and.pred q, e, g;\n\t"
+        "@q fence.proxy.async.shared::cta;\n\t"
+        "@q mbarrier.arrive.expect_tx.shared::cta.b64 _, [%1], 2048;\n\t"
+        "@q cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
+        "[%2], [%4, {%5, %6, %7}], [%1];\n\t"
+        "@q cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
+        "[%3], [%4, {%5, %6, 4}], [%1];\n\t}" ::"r"(static_cast<uint32_t>(go)),
+        "r"(bar), "r"(dst_u), "r"(dst_b), "l"(reinterpret_cast<uint64_t>(map)), "r"(col), "r"(row), "r"(zu)
+        : "memory");
+}
+
 // one TMA box {128 split columns, 1 row, 2 buffers}: the red and the black row of one
 // buffer pair, 1 KB, columns outside [0, ldh) and rows outside [0, n) zero-filled (those cells
 // are never written and only feed cells that are not)
@@ -340,9 +361,10 @@ __global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_
                 // refill: the slot row j+PF reuses was last read at step j-2 (u) / j-2 (b, row
                 // r+PF-RDB <= r-2T-1); all lanes are past step j-1 here
                 __syncwarp();
-                if (lane == 0 && j + PF < nsteps) {
-                    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
-                    issue(j + PF);
+                {
+                    const uint32_t cn = cc + PF;                              // counter of row j + PF
+                    refill_elected(j + PF < nsteps, smem_addr(&bars[cn % RDU]), smem_addr(ringU + (cn % RDU) * 256),
+                                   smem_addr(ringB + (cn % RDB) * 256), &p.tmap, kbase, r + PF, p.zu);
                 }
                 bar_wait(&bars[cc % RDU], (cc / RDU) & 1);
                 __syncwarp();
