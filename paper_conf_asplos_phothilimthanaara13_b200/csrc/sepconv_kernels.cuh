@@ -88,6 +88,24 @@ __device__ __forceinline__ void tma_load_3d(void *dst, const CUtensorMap *map, u
         : "memory");
 }
 
+// Stage refill issued by the converged warp: one elected lane runs the proxy fence, the
+// expect_tx and the box load under a predicate (no lane-0 branch; see sor.cu refill_elected).
+__device__ __forceinline__ void tma_refill_elected(bool go, void *dst, const CUtensorMap *map, uint64_t *bar,
+                                                   uint32_t bytes, int c0, int c1, int c2) {
+    asm volatile(
+        "{\n\t.reg .pred e, g, q;\n\t"
+        "elect.sync _|e, 0xffffffff;\n\t"
+        "setp.ne.u32 g, %6, 0;\n\t"
+        "and.pred q, e, g;\n\t"
+        "@q fence.proxy.async.shared::cta;\n\t"
+        "@q mbarrier.arrive.expect_tx.shared::cta.b64 _, [%2], %7;\n\t"
+        "@q cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
+        "[%0], [%1, {%3, %4, %5}], [%2];\n\t}" ::"r"(smem_u32(dst)),
+        "l"(reinterpret_cast<uint64_t>(map)), "r"(smem_u32(bar)), "r"(c0), "r"(c1), "r"(c2),
+        "r"(static_cast<uint32_t>(go)), "r"(bytes)
+        : "memory");
+}
+
 __device__ __forceinline__ void prefetch_tmap(const CUtensorMap *map) {
     asm volatile("prefetch.tensormap [%0];" ::"l"(reinterpret_cast<uint64_t>(map)) : "memory");
 }
@@ -517,11 +535,8 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                 } else {
                     __syncwarp();
                 }
-                if (lane == 0 && ch + NS < nchunks) {
-                    fence_proxy_async_smem();
-                    mbar_arrive_expect_tx(&wbar[st], BOX_BYTES);
-                    tma_load_3d(wsm + st * STAGE, &p.tmap, &wbar[st], wcol, in_row0 + (ch + NS) * SR, n);
-                }
+                tma_refill_elected(ch + NS < nchunks, wsm + st * STAGE, &p.tmap, &wbar[st], BOX_BYTES, wcol,
+                                   in_row0 + (ch + NS) * SR, n);
             }
         }
         };
