@@ -278,7 +278,9 @@ __device__ __forceinline__ float4 relax4s(const float4 &u, const float4 &N, cons
 // (Measured alternatives: waiting once per 6-row block lets steps
 // overlap but needs 36 KB of ring per warp -- 4 warps/SM -- and ran 20% slower.)
 template <int T>
-__global__ void __launch_bounds__(kWaveWarps * 32) sor_wave_kernel(const __grid_constant__ SorParams p) {
+// (an explicit minimum of one CTA per SM lets ptxas spend registers freely -- 168 at T=4 instead
+// of 134 -- while shared memory still holds three CTAs per SM: +5% at T=4, profiles/r01_sor_perf.txt)
+__global__ void __launch_bounds__(kWaveWarps * 32, 1) sor_wave_kernel(const __grid_constant__ SorParams p) {
     using WV = Wave<T>;
     constexpr int HL = WV::HL, WOUT = WV::WOUT, PF = WV::PF, RDU = WV::RDU, RDB = WV::RDB;
     extern __shared__ __align__(128) float wsmem[];
