@@ -60,6 +60,9 @@ def parse_args():
     ap.add_argument("--tune-reps", type=int, default=10)
     ap.add_argument("--sor-iters", type=int, default=24, help="poisson workload: iterations per step")
     ap.add_argument("--options", type=int, default=1 << 28, help="blackscholes workload: options per GPU")
+    ap.add_argument("--dry-run", action="store_true",
+                    help="launcher/protocol check without a GPU: N ranks on gloo exchange the halo rows of "
+                         "their bands (no convolution runs, value is null)")
     return ap.parse_args()
 
 
@@ -71,6 +74,42 @@ def peaks():
         return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs: torch D2D copy)"
     except Exception:
         return HBM_FALLBACK_GBS, "fallback (B200_PROFILING.md)"
+
+
+def _free_port() -> int:
+    import socket
+    with socket.socket(socket.AF_INET, socket.SOCK_STREAM) as so:
+        so.bind(("127.0.0.1", 0))
+        return so.getsockname()[1]
+
+
+def spawn_ranks(args):
+    """`bench.py --gpus N` outside torchrun: launch N ranks (one process per GPU) through
+    torch.distributed.run on 127.0.0.1 and return their exit status.  Never measures fewer
+    GPUs than asked: too few devices, or a WORLD_SIZE that disagrees with --gpus, is an error.
+    Returns None when this process is already the rank it should be."""
+    env_world = os.environ.get("WORLD_SIZE")
+    if env_world is not None:
+        if int(env_world) != args.gpus and args.impl != "reference":
+            print(f"[bench] error: --gpus {args.gpus} but WORLD_SIZE={env_world}", file=sys.stderr)
+            return 2
+        return None
+    if args.gpus <= 1 or args.impl == "reference":
+        return None
+    if not args.dry_run:
+        import torch
+        have = torch.cuda.device_count()
+        if have < args.gpus:
+            print(f"[bench] error: --gpus {args.gpus} but this node has {have} CUDA device(s)", file=sys.stderr)
+            return 2
+    env = dict(os.environ)
+    if not args.dry_run:                 # NCCL reports nranks when each communicator comes up
+        env.setdefault("NCCL_DEBUG", "INFO")
+        env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+           "--master-addr=127.0.0.1", f"--master-port={_free_port()}", os.path.abspath(__file__), *sys.argv[1:]]
+    print(f"[bench] launching {args.gpus} ranks: {' '.join(cmd)}", file=sys.stderr, flush=True)
+    return subprocess.call(cmd, env=env)
 
 
 def dist_env():
@@ -209,7 +248,8 @@ def run_reference(args):
            "image": [H, W], "images": 1 if args.workload == "image" else 64, "widths": widths,
            "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed, "sample": last["sample"],
            "parallelism": "host cores (oracle)"}
-    emit({"impl": "reference", "metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world,
+    emit({"impl": "reference", "metric": METRIC, "value": value, "unit": "Mpixels/s",
+          "n_gpus": world if world > 1 else args.gpus,
           "steps": args.steps, "warmup": args.warmup, "ms_per_step": statistics.median(times) * 1e3,
           "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
           "data": "synthetic", "config": cfg,
@@ -220,8 +260,65 @@ def run_reference(args):
 
 
 # --------------------------------------------------------------------------------------------
+def run_dry(args):
+    """--dry-run: the multi-rank plumbing of the image workload without a GPU.  Every rank takes
+    its row band from sepconv_band (host arithmetic of libsepconv.so), fills its owned input rows
+    from the seeded generator, receives the K-1 halo rows from rank g+1 over gloo (the exchange
+    sepconv_run_band does with NCCL) and checks them against the generator.  No convolution runs;
+    rank 0 prints the JSON line with value null."""
+    import torch
+    import torch.distributed as dist
+    from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+    world, rank, _ = dist_env()
+    if world > 1:
+        dist.init_process_group("gloo")
+    H = W = args.size
+    seed = synth.BENCH_SEED_BASE + 3
+    widths = [int(x) for x in args.widths.split(",")]
+    halo_ok = True
+    halo_bytes = 0
+    for K in widths:
+        r0, rows, owned, alloc = sc.band(H, K, world, rank)
+        band = np.zeros((alloc, W), np.float32)
+        band[:owned] = synth.uniform_image(H, W, seed, rows=(r0, r0 + owned))
+        if world > 1:
+            ops = []
+            if rank > 0:                            # my first K-1 rows are the predecessor's halo
+                ops.append(dist.P2POp(dist.isend, torch.from_numpy(np.ascontiguousarray(band[:K - 1])), rank - 1))
+            recv = torch.empty((alloc - owned, W), dtype=torch.float32)
+            if rank < world - 1 and alloc > owned:
+                ops.append(dist.P2POp(dist.irecv, recv, rank + 1))
+            for w_ in (dist.batch_isend_irecv(ops) if ops else []):
+                w_.wait()
+            if rank < world - 1 and alloc > owned:
+                band[owned:] = recv.numpy()
+                halo_bytes += recv.numel() * 4
+        want = synth.uniform_image(H, W, seed, rows=(r0, r0 + alloc))
+        halo_ok &= bool(np.array_equal(band, want))
+    flags = torch.tensor([0 if halo_ok else 1, halo_bytes], dtype=torch.int64)
+    if world > 1:
+        dist.all_reduce(flags)
+    if rank == 0:
+        emit({"metric": METRIC, "value": None, "unit": "Mpixels/s", "n_gpus": world, "steps": 0,
+              "warmup": 0, "ms_per_step": None, "higher_is_better": True, "scaling": "strong",
+              "vs_baseline": None, "dtype": "f32", "data": "synthetic", "dry_run": True,
+              "halo_exchange_ok": int(flags[0]) == 0, "halo_bytes": int(flags[1]),
+              "config": {"workload": f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, "
+                                     "one pass per width", "widths": widths,
+                         "parallelism": f"row bands x{world}, gloo halo send/recv (dry run)"}})
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+    return 0 if int(flags[0]) == 0 else 1
+
+
 def main():
     args = parse_args()
+    rc = spawn_ranks(args)
+    if rc is not None:
+        return rc
+    if args.dry_run:
+        return run_dry(args)
     if args.workload == "poisson":
         import bench_poisson
         return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit)
@@ -236,7 +333,9 @@ def main():
 
     world, rank, local = dist_env()
     if world != args.gpus:
-        print(f"[bench] warning: --gpus {args.gpus} but WORLD_SIZE={world}; using WORLD_SIZE", file=sys.stderr)
+        print(f"[bench] error: --gpus {args.gpus} but WORLD_SIZE={world}", file=sys.stderr)
+        return 2
+    print(f"[bench] rank {rank}/{world} on cuda:{local}", file=sys.stderr, flush=True)
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
     dist = None

@@ -49,7 +49,8 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
             if i >= args.warmup:
                 vals.append(last["value"])
         v = statistics.median(vals)
-        emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Moptions/s", "n_gpus": world,
+        emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Moptions/s",
+              "n_gpus": world if world > 1 else args.gpus,
               "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "weak",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
               "config": {"workload": (f"Black-Scholes, {args.options} float32 options per GPU "

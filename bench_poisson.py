@@ -51,7 +51,8 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
             if i >= args.warmup:
                 vals.append(last["value"])
         v = statistics.median(vals)
-        emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Mcell-it/s", "n_gpus": world,
+        emit({"impl": "reference", "metric": METRIC, "value": v, "unit": "Mcell-it/s",
+              "n_gpus": world if world > 1 else args.gpus,
               "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
               "config": {"workload": (f"Poisson2D red-black SOR, {args.size}x{args.size} float32 grid, "

@@ -66,7 +66,7 @@ def _load():
             lib.oracle_rb_merge.argtypes = [f32p, f32p, i64, i64, f32p]
             lib.oracle_poisson_residual.argtypes = [f64p, f32p, i64, i64, f64p]
             lib.oracle_black_scholes.argtypes = [f32p, f32p, f32p, i64, ctypes.c_double, ctypes.c_double,
-                                                 f64p, f64p, ctypes.c_void_p]
+                                                 f64p, f64p, ctypes.c_void_p, ctypes.c_void_p]
             for fn in (lib.oracle_convolve2d, lib.oracle_convolve_rows,
                        lib.oracle_convolve_columns, lib.oracle_separable, lib.oracle_num_cpus,
                        lib.oracle_sor_rb, lib.oracle_sor_rb_f32, lib.oracle_rb_split,
@@ -263,15 +263,18 @@ def sor_abs_scale(x, b, omega: float, iters: int):
 # ---- Black-Scholes (blackscholes.c) -----------------------
 def black_scholes(s, x, t, r: float, v: float, with_scale: bool = False):
     """European call and put prices in double for float32 spot s, strike x, expiry t (years)
-    and scalar rate r, volatility v; optionally the float32 error scale of reading B4."""
+    and scalar rate r, volatility v.  With ``with_scale`` also the float32 error scales of the
+    call and of the put (reading B4): returns (call, put, scale_call, scale_put)."""
     s, x, t = (np.ascontiguousarray(np.asarray(a, np.float32).reshape(-1)) for a in (s, x, t))
     if not (s.size == x.size == t.size):
         raise ValueError("s, x, t differ in length")
     call = np.empty(s.size, np.float64)
     put = np.empty(s.size, np.float64)
-    scale = np.empty(s.size, np.float64) if with_scale else None
+    sc = np.empty(s.size, np.float64) if with_scale else None
+    sp = np.empty(s.size, np.float64) if with_scale else None
     rc = _load().oracle_black_scholes(s, x, t, s.size, float(r), float(v), call, put,
-                                      scale.ctypes.data if with_scale else None)
+                                      sc.ctypes.data if with_scale else None,
+                                      sp.ctypes.data if with_scale else None)
     if rc != 0:
         raise ValueError("oracle_black_scholes rejected its arguments")
-    return (call, put, scale) if with_scale else (call, put)
+    return (call, put, sc, sp) if with_scale else (call, put)

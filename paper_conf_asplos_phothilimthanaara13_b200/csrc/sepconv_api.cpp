@@ -163,9 +163,8 @@ static sepconv_status_t make_tmap(sepconv_plan_t plan, CUtensorMap *map, const f
                                   int nimg, long long ld, long long img, int box_w, int box_h) {
     EncodeTiledFn enc = encode_fn();
     if (!enc) return fail(SEPCONV_E_CUDA, "cuTensorMapEncodeTiled unavailable from the driver");
-    const long long key2 = ((((static_cast<long long>(cols) * 1315423911LL + rows) * 2654435761LL + nimg) * 97 + ld) *
-                                31 + img) * 131 + box_w * 1024 + box_h;
-    auto key = std::make_pair(reinterpret_cast<uintptr_t>(base), key2);
+    const std::array<long long, 8> key{static_cast<long long>(reinterpret_cast<uintptr_t>(base)), cols, rows, nimg,
+                                       ld, img, box_w, box_h};
     auto it = plan->tmaps.maps.find(key);
     if (it != plan->tmaps.maps.end()) {
         *map = it->second;

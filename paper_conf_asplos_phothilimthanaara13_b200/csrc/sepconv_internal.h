@@ -3,6 +3,7 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <array>
 #include <atomic>
 #include <cstdarg>
 #include <cstdint>
@@ -53,7 +54,10 @@ struct Candidate {
 };
 
 struct TensorMapCache {
-    std::map<std::pair<uintptr_t, long long>, CUtensorMap> maps;   // key: (base, shape hash)
+    // key: every field the encoded map depends on -- (base, cols, rows, images, ld, image
+    // stride, box width, box height) -- compared exactly, so two geometries on one base (band
+    // interior / tail, the unfused ROWS pass's shifted pointer) never share a map
+    std::map<std::array<long long, 8>, CUtensorMap> maps;
 };
 
 struct DeviceInfo {

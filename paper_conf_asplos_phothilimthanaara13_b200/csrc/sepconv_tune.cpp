@@ -8,6 +8,9 @@
 // the fastest of each algorithm becomes 2D's / SEPARABLE's.  Ties within 1% prefer
 // fewer passes, then the lower candidate index (R17).
 #include <cuda_runtime.h>
+#include <fcntl.h>
+#include <sys/file.h>
+#include <unistd.h>
 
 #include <algorithm>
 #include <cmath>
@@ -17,6 +20,7 @@
 #include <fstream>
 #include <sstream>
 #include <string>
+#include <thread>
 #include <vector>
 
 #include "sepconv_internal.h"
@@ -97,7 +101,26 @@ bool load_cache(const std::string &path, const std::string &key, sepconv_choice_
     return found;
 }
 
-void store_cache(const std::string &path, const std::string &key, const sepconv_choice_t best[3]) {
+// Read-modify-write of the JSON-lines cache under an exclusive flock on "<path>.lock", through a
+// temp file unique to this process and thread, then an atomic rename: several ranks or
+// processes sharing one cache (multi-GPU bench runs) neither truncate each other's temp file
+// nor lose each other's entries.
+struct CacheLock {
+    int fd = -1;
+    explicit CacheLock(const std::string &path) {
+        fd = ::open((path + ".lock").c_str(), O_RDWR | O_CREAT | O_CLOEXEC, 0644);
+        if (fd >= 0) ::flock(fd, LOCK_EX);
+    }
+    ~CacheLock() {
+        if (fd >= 0) {
+            ::flock(fd, LOCK_UN);
+            ::close(fd);
+        }
+    }
+};
+
+void store_cache(const std::string &path, const std::string &key, const std::string &entry) {
+    CacheLock lock(path);
     std::vector<std::string> keep;
     {
         std::ifstream f(path);
@@ -105,14 +128,26 @@ void store_cache(const std::string &path, const std::string &key, const sepconv_
         while (f && std::getline(f, line))
             if (!line.empty() && line.find(want) == std::string::npos) keep.push_back(line);
     }
-    std::string tmp = path + ".tmp";
-    std::ofstream o(tmp, std::ios::trunc);
-    if (!o) return;
-    for (auto &l : keep) o << l << "\n";
-    o << "{\"key\":\"" << key << "\",\"2d\":" << choice_json(best[0]) << ",\"sep\":" << choice_json(best[1])
-      << ",\"auto\":" << choice_json(best[2]) << "}\n";
-    o.close();
-    std::rename(tmp.c_str(), path.c_str());
+    std::ostringstream tn;
+    tn << path << ".tmp." << ::getpid() << "." << std::hash<std::thread::id>{}(std::this_thread::get_id());
+    const std::string tmp = tn.str();
+    {
+        std::ofstream o(tmp, std::ios::trunc);
+        if (!o) return;
+        for (auto &l : keep) o << l << "\n";
+        o << entry << "\n";
+        if (!o.good()) {
+            o.close();
+            std::remove(tmp.c_str());
+            return;
+        }
+    }
+    if (std::rename(tmp.c_str(), path.c_str()) != 0) std::remove(tmp.c_str());
+}
+
+void store_choices(const std::string &path, const std::string &key, const sepconv_choice_t best[3]) {
+    store_cache(path, key, "{\"key\":\"" + key + "\",\"2d\":" + choice_json(best[0]) + ",\"sep\":" +
+                               choice_json(best[1]) + ",\"auto\":" + choice_json(best[2]) + "}");
 }
 
 // The paper's selector picks a rule by input-size cutoffs (SELECT).  Here: a
@@ -296,7 +331,7 @@ sepconv_status_t sepconv_tune(sepconv_plan_t plan, const sepconv_tune_opts_t *op
         o.median_us = med[bi[s]];
     }
     plan->tuned = true;
-    if (!path.empty()) store_cache(path, key, plan->best);
+    if (!path.empty()) store_choices(path, key, plan->best);
     if (chosen) *chosen = plan->best[2];
     return SEPCONV_OK;
 }

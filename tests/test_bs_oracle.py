@@ -87,10 +87,12 @@ def test_monotone_in_spot_strike_and_volatility():
 
 def test_error_scale_bounds_a_float32_evaluation():
     """A float32 evaluation of the same formula (numpy, float32 throughout, erfc from
-    math in double then rounded) stays within 16 eps x the oracle's B4 error scale."""
-    s, x, t = synth.bs_options(2000, seed=9)
+    math in double then rounded) stays within 16 eps x the oracle's B4 error scales, and the
+    bound is TIGHT: the observed error reaches >= 2% of it for the call and for the put (an
+    inflated scale would fail here)."""
+    s, x, t = synth.bs_options(20000, seed=9)
     r, v = np.float32(synth.BS_RATE), np.float32(synth.BS_VOL)
-    c, p, scale = oracle.black_scholes(s, x, t, float(r), float(v), with_scale=True)
+    c, p, sc_c, sc_p = oracle.black_scholes(s, x, t, float(r), float(v), with_scale=True)
     sq = np.sqrt(t)
     d1 = (np.log(s / x) + (r + np.float32(0.5) * v * v) * t) / (v * sq)
     d2 = d1 - v * sq
@@ -99,8 +101,28 @@ def test_error_scale_bounds_a_float32_evaluation():
     c32 = s * n(d1) - disc * n(d2)
     p32 = disc * n(-d2) - s * n(-d1)
     eps = 2.0 ** -24
-    assert np.all(np.abs(c32 - c) <= 16 * eps * scale)
-    assert np.all(np.abs(p32 - p) <= 16 * eps * scale)
+    assert np.all(np.abs(c32 - c) <= 16 * eps * sc_c)
+    assert np.all(np.abs(p32 - p) <= 16 * eps * sc_p)
+    assert np.max(np.abs(c32 - c) / (16 * eps * sc_c)) >= 0.02
+    assert np.max(np.abs(p32 - p) / (16 * eps * sc_p)) >= 0.02
+
+
+def test_error_scale_is_relative_to_the_price():
+    """Upper pin of reading B4: the tolerance 16 eps x scale is a small fraction of the price
+    itself at moneyness S/X in [0.5, 2] (<= 1%), including out-of-the-money options whose price
+    is far below S -- an absolute allowance of a few ulps of S would exceed their price.  And a
+    deep out-of-the-money call (S = 1, X = 1000: price ~1e-190) is held to ~1e-33, not
+    to ulps of S (a few FLT_MIN x (S + X), reading B3)."""
+    s, x, t = synth.bs_options(20000, seed=9)
+    c, p, sc_c, sc_p = oracle.black_scholes(s, x, t, synth.BS_RATE, synth.BS_VOL, with_scale=True)
+    eps = 2.0 ** -24
+    m = s.astype(np.float64) / x
+    sel = (m >= 0.5) & (m <= 2.0)
+    assert sel.sum() > 1000
+    assert np.max(16 * eps * sc_c[sel] / c[sel]) <= 0.01
+    assert np.max(16 * eps * sc_p[sel] / p[sel]) <= 0.01
+    c1, _, s1, _ = oracle.black_scholes([1.0], [1000.0], [1.0], 0.03, 0.2, with_scale=True)
+    assert 16 * eps * s1[0] <= 1e-30 and c1[0] < 1e-100
 
 
 def test_rejects_invalid_inputs():

@@ -110,8 +110,8 @@ def test_random_black_scholes_configuration(seed):
     dev[4].fill_(float("nan"))
     bs.price(dev[0][off:], dev[1][off:], dev[2][off:], r, v, dev[3][off:], dev[4][off:], n=n)
     torch.cuda.synchronize()
-    oc, op, scale = oracle.black_scholes(s, x, t, r, v, with_scale=True)
-    for got, want in ((dev[3][off:], oc), (dev[4][off:], op)):
+    oc, op, sc_c, sc_p = oracle.black_scholes(s, x, t, r, v, with_scale=True)
+    for got, want, scale in ((dev[3][off:], oc, sc_c), (dev[4][off:], op, sc_p)):
         g = got.cpu().numpy()
         assert not np.any(np.isnan(g))
         assert np.all(np.abs(g - want) <= 16 * 2.0 ** -24 * scale)
