@@ -425,12 +425,17 @@ def main():
     ev = {K: [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
               for _ in range(args.steps)] for K in widths}
     e_start, e_end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    # working sets that fit in L2 (in + out <= 2 x L2) are flushed before every pass by writing a
-    # scratch buffer of 2 x L2 (a torch fill, outside the per-pass events), and ms_per_step is then
-    # the sum of the per-pass device times; larger inputs stream from HBM anyway (no flush)
+    # working sets that fit in L2 (in + out <= 2 x L2) are flushed before every pass, outside the
+    # per-pass events: a write of a 2 x L2 scratch buffer, then a read of a second 2 x L2 buffer so
+    # the pass starts from an L2 of clean, unrelated lines (a write alone leaves ~L2-size of dirty
+    # lines whose write-back the timed pass would pay: +2-6 us at 2048^2-4096^2,
+    # profiles/r02_flush_study.txt); ms_per_step is then the sum of the per-pass device times.
+    # Larger inputs stream from HBM anyway (no flush).
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
     scratch = torch.empty(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
+    rscratch = torch.zeros(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
+    sink = torch.empty((), dtype=torch.float32, device=dev)
     launches0 = sc.launch_count()
     with ClockSampler(local) as clk:
         torch.cuda.synchronize()
@@ -442,6 +447,7 @@ def main():
             for K in widths:
                 if flush:
                     scratch.fill_(float(s))
+                    torch.sum(rscratch, dim=0, out=sink)
                 ev[K][s][0].record(stream)
                 one_pass(K)
                 ev[K][s][1].record(stream)
@@ -496,7 +502,8 @@ def main():
     if os.path.exists(tr_path):
         try:
             tr = json.load(open(tr_path))
-            vals = [tr[f"{dom}:K{K}"] for K in dom_k if f"{dom}:K{K}" in tr and args.workload == "image"
+            base = dom.split("@")[0]                       # ncu traffic is per candidate, any schedule
+            vals = [tr[f"{base}:K{K}"] for K in dom_k if f"{base}:K{K}" in tr and args.workload == "image"
                     and world == 1 and H == 16384]
             if len(vals) == len(dom_k):
                 traffic = sum(vals) / len(vals)
@@ -586,8 +593,9 @@ def main():
                             if args.workload == "image" else f"{N_img} x {H}x{W} float32 images, width 11"),
                "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
                "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
-               "l2": ("L2 flushed before every pass (2 x L2 write, outside the per-pass events; "
-                      "ms_per_step = sum of per-pass device times)") if flush else "inputs larger than L2 (no flush)",
+               "l2": ("L2 flushed before every pass (write 2 x L2, then read another 2 x L2 so L2 holds clean "
+                      "unrelated lines; outside the per-pass events; ms_per_step = sum of per-pass device times)")
+               if flush else "inputs larger than L2 (no flush)",
                "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
                                else f"images sharded x{world}" if world > 1 else "1 GPU")}
         emit({"metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world, "steps": args.steps,

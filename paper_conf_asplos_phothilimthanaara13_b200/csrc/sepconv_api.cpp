@@ -13,6 +13,7 @@
 #include <mutex>
 #include <new>
 #include <string>
+#include <vector>
 
 #include "sepconv_internal.h"
 
@@ -204,10 +205,6 @@ static bool tma_ok(const float *base, long long ld, long long img) {
 // and the e = slots - q*S leftover CTAs share the short last window, m = ceil(S/e)
 // segments each; P solves P + o = m*(rows - q*P + o) (o = per-segment overhead in rows).
 // $SEPCONV_SCHED = "nowin" disables it, "win" forces it where eligible (tests, A/B runs).
-struct Sched {
-    int grid, parts, win_rows, extra;
-};
-
 static Sched schedule_uncached(long long slots, int nimg, int nstrips, int rows, int K, bool no_win, bool force_win) {
     const long long strips = static_cast<long long>(nimg) * nstrips;
     // segments may be short: the score below already charges each one its K-1 warm-up rows,
@@ -287,12 +284,26 @@ static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int 
     return sc;
 }
 
+// A tuner-mutated schedule (sepconv_choice_t.sched_parts / sched_grid) replaces the model's:
+// `parts` strided row partitions per (image, strip) over `grid` CTAs, both clamped to what the
+// geometry and the resident slots allow.  Any (parts, grid) is a valid SegmentIter schedule.
+static Sched apply_override(const Sched &model, long long slots, int nimg, int nstrips, int rows, int parts,
+                            int grid) {
+    if (parts <= 0) return model;
+    const long long p = std::max(1, std::min(parts, rows));
+    const long long items = static_cast<long long>(nimg) * nstrips * p;
+    long long g = grid > 0 ? grid : slots;
+    g = std::max<long long>(1, std::min(std::min(g, slots), items));
+    return Sched{static_cast<int>(g), static_cast<int>(p), 0, 0};
+}
+
 // One streaming pass (ROWS, COLS or SEP) over geometry g.
 static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geometry &g, const float *in,
                                          long long ld_in, long long in_img, int in_cols, float *out,
                                          long long ld_out, long long out_img, int out_cols, int rows_total,
                                          const float *kernel, bool want_tma, int cfg, int store_path,
-                                         cudaStream_t st) {
+                                         cudaStream_t st, int ov_parts = 0, int ov_grid = 0,
+                                         Sched *query = nullptr, long long *query_slots = nullptr) {
     const int K = g.K;
     const bool tma = want_tma && tma_ok(in, ld_in, in_img);
     const bool vec = aligned(in, 16) && (ld_in % 4) == 0 && (in_img % 4) == 0;
@@ -330,12 +341,19 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
         p.k[i] = kernel[i];
         p.k2[i] = make_float2(kernel[i], kernel[i]);
     }
-    if (tma) {
+    if (tma && !query) {
         s = make_tmap(plan, &p.tmap, in, in_cols, g.in_rows, g.nimg, ld_in, in_img, stream_bw(K, op), ki.stage_rows);
         if (s != SEPCONV_OK) return s;
     }
+    const long long slots = static_cast<long long>(plan->dev.sms) * occ;
+    const Sched sc = apply_override(schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K), slots, g.nimg,
+                                    p.nstrips, rows_total, ov_parts, ov_grid);
+    if (query) {                                               // candidate_sched: report, do not launch
+        *query = sc;
+        if (query_slots) *query_slots = slots;
+        return SEPCONV_OK;
+    }
     if (p.total <= 0) return SEPCONV_OK;
-    const Sched sc = schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K);
     p.parts = sc.parts;
     p.win_rows = sc.win_rows;
     p.extra = sc.extra;
@@ -346,7 +364,8 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
 }
 
 static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const float *in, float *out,
-                                  const float *kernel, bool want_tma, cudaStream_t st) {
+                                  const float *kernel, bool want_tma, cudaStream_t st, int ov_parts = 0,
+                                  int ov_grid = 0, Sched *query = nullptr, long long *query_slots = nullptr) {
     const int K = g.K;
     const bool tma = want_tma && tma_ok(in, g.ld_in, g.in_img);
     const bool vec = aligned(in, 16) && (g.ld_in % 4) == 0 && (g.in_img % 4) == 0;
@@ -376,13 +395,20 @@ static sepconv_status_t launch_2d(sepconv_plan_t plan, const Geometry &g, const 
     // w_ji = fl(k_i * k_j): the outer-product weights of Convolve2D, rounded once
     for (int j = 0; j < K; ++j)
         for (int i = 0; i < K; ++i) p.w[j * K + i] = kernel[i] * kernel[j];
-    if (tma) {
+    if (tma && !query) {
         s = make_tmap(plan, &p.tmap, in, g.in_cols, g.in_rows, g.nimg, g.ld_in, g.in_img, box_width(K, true),
                       Conv2DCfg<1>::SR);
         if (s != SEPCONV_OK) return s;
     }
+    const long long slots = static_cast<long long>(plan->dev.sms) * occ;
+    const Sched sc = apply_override(schedule(plan->dev, occ, g.nimg, p.nstrips, g.rows, K), slots, g.nimg, p.nstrips,
+                                    g.rows, ov_parts, ov_grid);
+    if (query) {
+        *query = sc;
+        if (query_slots) *query_slots = slots;
+        return SEPCONV_OK;
+    }
     if (p.total <= 0) return SEPCONV_OK;
-    const Sched sc = schedule(plan->dev, occ, g.nimg, p.nstrips, g.rows, K);
     p.parts = sc.parts;
     p.win_rows = sc.win_rows;
     p.extra = sc.extra;
@@ -408,10 +434,14 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
                                   const float *kernel, const Candidate &c, float *buf, long long ld_buf,
                                   cudaStream_t st) {
     const bool tma = c.mapping == SEPCONV_MAP_TMA;
-    if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st);
+    // a schedule override was tuned for the plan's whole geometry; bands and host-pipeline
+    // chunks (other row counts) use the model
+    const bool whole = g.row_begin == 0 && g.rows == plan->ho && g.nimg == plan->n;
+    const int ovp = whole ? c.sched_parts : 0, ovg = whole ? c.sched_grid : 0;
+    if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st, ovp, ovg);
     if (c.fused)
         return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, c.config, c.store, st);
+                                g.out_cols, g.rows, kernel, tma, c.config, c.store, st, ovp, ovg);
     // Choice 2 as the paper writes it: ConvolveRows into buffer, then ConvolveColumns.
     // The buffer holds the rows this launch's output rows need: [row_begin, row_begin + rows + K - 1).
     if (!buf) return fail(SEPCONV_E_INVALID, "unfused separable needs a workspace");
@@ -442,6 +472,44 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
     }
 }
 
+sepconv_status_t candidate_sched(sepconv_plan_t plan, const Geometry &g, const Candidate &c, Sched *sc,
+                                 long long *slots) {
+    // the same pointers' alignment as the tuner's buffers (cudaMalloc: 256-byte aligned)
+    const float *in = reinterpret_cast<const float *>(uintptr_t{256});
+    float *out = reinterpret_cast<float *>(uintptr_t{512});
+    const bool tma = c.mapping == SEPCONV_MAP_TMA;
+    std::vector<float> k(g.K, 0.f);
+    if (c.algo == SEPCONV_2D)
+        return launch_2d(plan, g, in, out, k.data(), tma, nullptr, c.sched_parts, c.sched_grid, sc, slots);
+    if (!c.fused) return fail(SEPCONV_E_INVALID, "candidate_sched: the unfused pair has two schedules");
+    return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img, g.out_cols,
+                            g.rows, k.data(), tma, c.config, c.store, nullptr, c.sched_parts, c.sched_grid, sc, slots);
+}
+
+Candidate from_choice(const sepconv_choice_t &c) {
+    Candidate r{static_cast<int>(c.algo), c.mapping, c.algo == SEPCONV_SEPARABLE ? c.fused : 0, c.config,
+                c.store_path};
+    r.sched_parts = c.sched_parts;
+    r.sched_grid = c.sched_grid;
+    return r;
+}
+
+sepconv_choice_t to_choice(const Candidate &c, int K, int source) {
+    sepconv_choice_t o;
+    std::memset(&o, 0, sizeof o);
+    o.algo = static_cast<sepconv_variant_t>(c.algo);
+    o.mapping = c.mapping;
+    o.fused = c.fused;
+    o.config = c.config;
+    o.store_path = c.store;
+    o.warps = candidate_warps(K, c);
+    o.ctas_per_sm = 1;
+    o.sched_parts = c.sched_parts;
+    o.sched_grid = c.sched_grid;
+    o.source = source;
+    return o;
+}
+
 // Static default before tuning (R16): fused separable with TMA for K >= 2
 // (one HBM pass, 2K FMA/px), 2D with TMA for K = 1.
 static Candidate default_candidate(int K, sepconv_variant_t v) {
@@ -457,10 +525,7 @@ int candidate_warps(int K, const Candidate &c) {
 
 Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v) {
     const int idx = v == SEPCONV_2D ? 0 : v == SEPCONV_SEPARABLE ? 1 : 2;
-    if (plan->tuned) {
-        const sepconv_choice_t &c = plan->best[idx];
-        return {static_cast<int>(c.algo), c.mapping, c.fused, c.config, c.store_path};
-    }
+    if (plan->tuned) return from_choice(plan->best[idx]);
     return default_candidate(plan->k, v);
 }
 
@@ -601,6 +666,8 @@ static sepconv_status_t check_choice(const sepconv_choice_t *c) {
     if (c->config < 0 || c->config >= kSepTmaConfigs)
         return fail(SEPCONV_E_INVALID, "choice.config must be in [0, %d)", kSepTmaConfigs);
     if (c->store_path < 0 || c->store_path > 1) return fail(SEPCONV_E_INVALID, "choice.store_path must be 0 or 1");
+    if (c->sched_parts < 0 || c->sched_grid < 0)
+        return fail(SEPCONV_E_INVALID, "choice.sched_parts / sched_grid must be >= 0");
     return SEPCONV_OK;
 }
 
@@ -638,9 +705,7 @@ sepconv_status_t sepconv_run_choice(sepconv_plan_t plan, const float *in, const 
     if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
     sepconv_status_t s = check_choice(choice);
     if (s != SEPCONV_OK) return s;
-    Candidate c{static_cast<int>(choice->algo), choice->mapping, choice->algo == SEPCONV_SEPARABLE ? choice->fused : 0,
-                choice->config, choice->store_path};
-    return run_resolved(plan, in, kernel, out, c, static_cast<cudaStream_t>(stream));
+    return run_resolved(plan, in, kernel, out, from_choice(*choice), static_cast<cudaStream_t>(stream));
 }
 
 sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t variant, sepconv_choice_t *choice) {
@@ -649,19 +714,8 @@ sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t varia
     if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
         return fail(SEPCONV_E_INVALID, "bad variant");
     const int idx = variant == SEPCONV_2D ? 0 : variant == SEPCONV_SEPARABLE ? 1 : 2;
-    if (plan->tuned) {
-        *choice = plan->best[idx];
-    } else {
-        Candidate c = resolve(plan, variant);
-        std::memset(choice, 0, sizeof *choice);
-        choice->algo = static_cast<sepconv_variant_t>(c.algo);
-        choice->mapping = c.mapping;
-        choice->fused = c.fused;
-        choice->config = c.config;
-        choice->store_path = c.store;
-        choice->warps = candidate_warps(plan->k, c);
-        choice->ctas_per_sm = 1;
-    }
+    if (plan->tuned) *choice = plan->best[idx];
+    else *choice = to_choice(resolve(plan, variant), plan->k, SEPCONV_SRC_DEFAULT);
     return SEPCONV_OK;
 }
 

@@ -51,6 +51,14 @@ struct Candidate {
     int fused;     // separable only
     int config;    // fused + TMA: stage configuration 0..kSepTmaConfigs-1 (stream_geom)
     int store;     // 0: 16-byte store path when every output row allows it, 1: always the 8-byte path
+    int sched_parts = 0;   // work-schedule override (sepconv_choice_t.sched_parts): 0 = model
+    int sched_grid = 0;    // CTAs of the override (0 = every resident slot)
+};
+
+// The work schedule a launch uses (SegmentIter, sepconv_kernels.cuh): grid CTAs; parts > 0
+// strided row partitions, 0 contiguous, -q the window schedule (win_rows, extra).
+struct Sched {
+    int grid, parts, win_rows, extra;
 };
 
 struct TensorMapCache {
@@ -82,7 +90,8 @@ struct sepconv_plan_s {
     int64_t ld_buf = 0;
     size_t buf_floats = 0;
 
-    // tuned choices: [0] 2D, [1] SEPARABLE, [2] AUTO
+    // tuned choices: [0] 2D, [1] SEPARABLE, [2] AUTO; best[i].source says where each came
+    // from (tuned on this shape, or SELECT over a size selector)
     bool tuned = false;
     sepconv_choice_t best[3] = {};
 
@@ -111,6 +120,12 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
                                   const float *kernel, const Candidate &c, float *buf, long long ld_buf,
                                   cudaStream_t st);
 Candidate resolve(sepconv_plan_t plan, sepconv_variant_t v);
+// the schedule launch_candidate would give c on geometry g (model or override) and the
+// resident-slot count it was sized for; single-kernel candidates only (fused, 2D)
+sepconv_status_t candidate_sched(sepconv_plan_t plan, const Geometry &g, const Candidate &c, Sched *sc,
+                                 long long *slots);
+Candidate from_choice(const sepconv_choice_t &c);
+sepconv_choice_t to_choice(const Candidate &c, int K, int source);
 int candidate_warps(int K, const Candidate &c);
 sepconv_status_t check_kernel(const float *kernel, int K);
 Geometry plan_geometry(sepconv_plan_t plan);

@@ -34,5 +34,7 @@ cudaError_t conv2d_launch(int map, int K, const Conv2DParams &p, int grid, cudaS
 // utility kernels (sepconv_util.cu)
 cudaError_t launch_fill_pattern(float *dst, long long n, unsigned seed, cudaStream_t st);
 cudaError_t launch_l2_flush(float *scratch, long long n, cudaStream_t st);
+// read a second buffer of >= 2 x L2 (zero-filled by the caller) after launch_l2_flush: L2 ends clean
+cudaError_t launch_l2_clean(const float *src, long long n, float *sink, cudaStream_t st);
 
 }  // namespace sepconv

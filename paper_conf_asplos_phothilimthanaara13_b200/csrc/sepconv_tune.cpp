@@ -1,12 +1,26 @@
-// sepconv_tune.cpp -- the empirical tuner (the paper's autotuner, reduced to
-// an exhaustive search: the B200 space is a handful of candidates per plan, so
-// timing every one is exact where the paper needed evolutionary search).
+// sepconv_tune.cpp -- the empirical tuner (the paper's autotuner) and its size
+// selector (SELECT).
 //
-// For each eligible candidate: warm up, then `reps` timed runs with CUDA events on a
-// private stream, the L2 flushed before each run when the working set would fit in L2
-// (the same hygiene as bench.py), median.  The fastest overall becomes AUTO's choice,
-// the fastest of each algorithm becomes 2D's / SEPARABLE's.  Ties within 1% prefer
-// fewer passes, then the lower candidate index (R17).
+// sepconv_tune(plan): every eligible candidate (compile-time stage configurations, store
+// paths, mappings, algorithms) is timed -- the B200 space is a handful of candidates per plan,
+// so the exhaustive pass is exact where the paper needed an evolutionary search -- then the
+// winner's work schedule, a pair of size-like integers (row partitions per CTA strip, CTAs),
+// goes through the paper's mutation search: one parent, asexual children made by
+// scaling the values by lognormal factors (a halving as likely as a doubling, small changes
+// likelier than large ones), a child kept only if it beats its parent.
+// The fastest overall becomes AUTO's choice, the fastest of each algorithm 2D's / SEPARABLE's.
+// Ties within 1% prefer fewer passes, then the lower candidate index (R17).
+//
+// Timing: when in + out fit in 2 x L2 every timed pass follows a clean
+// flush -- a write of 2 x L2 then a read of another 2 x L2, so the pass pays for its own
+// traffic and not for write-backs of lines an unrelated kernel dirtied -- and the pass time is
+// the event time of n x (flush + pass) minus that of n x (flush), because single events tick
+// in 2.048 us steps on this system (profiles/r02_flush_study.txt); larger working sets time n
+// back-to-back passes.  The result is the median of three such batches.
+//
+// sepconv_tune_selector(K): the exhaustive tuner at up to 12 square sizes, equal neighbouring
+// picks merged, each cutoff between different picks placed by timing both at the geometric
+// middle; stored in the cache so that plans of untuned shapes resolve AUTO by SELECT.
 #include <cuda_runtime.h>
 #include <fcntl.h>
 #include <sys/file.h>
@@ -18,9 +32,11 @@
 #include <cstdlib>
 #include <cstring>
 #include <fstream>
+#include <functional>
 #include <sstream>
 #include <string>
 #include <thread>
+#include <tuple>
 #include <vector>
 
 #include "sepconv_internal.h"
@@ -48,32 +64,37 @@ std::vector<Candidate> candidates(sepconv_plan_t p) {
 
 int passes(const Candidate &c) { return (c.algo == SEPCONV_SEPARABLE && !c.fused) ? 2 : 1; }
 
-std::string cache_key(sepconv_plan_t p) {
+std::string plan_key(sepconv_plan_t p) {
     std::ostringstream os;
     os << p->dev.name << "|" << p->dev.sms << "|" << p->n << "x" << p->h << "x" << p->w << "|k" << p->k << "|ld"
        << p->ld_in << "," << p->ld_out;
     return os.str();
 }
 
+std::string selector_key(const DeviceInfo &d, int K) {
+    std::ostringstream os;
+    os << "sel:" << d.name << "|" << d.sms << "|k" << K;
+    return os.str();
+}
+
+// ---- the JSON-lines cache -------------------------------------------------------------------
 std::string choice_json(const sepconv_choice_t &c) {
-    char b[160];
-    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g]", (int)c.algo, c.mapping, c.fused, c.config, c.store_path,
-             c.warps, c.ctas_per_sm, c.median_us);
+    char b[200];
+    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g,%d,%d]", (int)c.algo, c.mapping, c.fused, c.config,
+             c.store_path, c.warps, c.ctas_per_sm, c.median_us, c.sched_parts, c.sched_grid);
     return b;
 }
 
-bool parse_choice(const std::string &line, const char *field, sepconv_choice_t *c) {
-    std::string f = std::string("\"") + field + "\":[";
-    size_t pos = line.find(f);
-    if (pos == std::string::npos) return false;
-    int algo, map, fused, config, store, warps, ctas;
+// parses one "[...]" choice at p; returns the position after it, or nullptr
+const char *parse_choice_at(const char *p, sepconv_choice_t *c) {
+    int algo, map, fused, config, store, warps, ctas, parts = 0, grid = 0, used = 0;
     float us;
-    if (sscanf(line.c_str() + pos + f.size(), "%d,%d,%d,%d,%d,%d,%d,%f", &algo, &map, &fused, &config, &store, &warps,
-               &ctas, &us) != 8)
-        return false;
-    if (store < 0 || store > 1) return false;
-    if (config < 0 || config >= kSepTmaConfigs) return false;
-    if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return false;
+    if (sscanf(p, "[%d,%d,%d,%d,%d,%d,%d,%f,%d,%d]%n", &algo, &map, &fused, &config, &store, &warps, &ctas, &us, &parts,
+               &grid, &used) != 10 || used == 0)
+        return nullptr;
+    if (store < 0 || store > 1 || config < 0 || config >= kSepTmaConfigs || parts < 0 || grid < 0) return nullptr;
+    if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return nullptr;
+    std::memset(c, 0, sizeof *c);
     c->algo = static_cast<sepconv_variant_t>(algo);
     c->mapping = map;
     c->fused = fused;
@@ -82,23 +103,41 @@ bool parse_choice(const std::string &line, const char *field, sepconv_choice_t *
     c->warps = warps;
     c->ctas_per_sm = ctas;
     c->median_us = us;
-    return true;
+    c->sched_parts = parts;
+    c->sched_grid = grid;
+    return p + used;
 }
 
-bool load_cache(const std::string &path, const std::string &key, sepconv_choice_t best[3]) {
+bool parse_choice(const std::string &line, const char *field, sepconv_choice_t *c) {
+    const std::string f = std::string("\"") + field + "\":";
+    const size_t pos = line.find(f);
+    return pos != std::string::npos && parse_choice_at(line.c_str() + pos + f.size(), c) != nullptr;
+}
+
+// the last line of the cache whose key is exactly `key`
+bool find_line(const std::string &path, const std::string &key, std::string *out) {
     std::ifstream f(path);
     if (!f) return false;
-    std::string line, want = "\"key\":\"" + key + "\"";
+    const std::string want = "{\"key\":\"" + key + "\",";
+    std::string line;
     bool found = false;
-    while (std::getline(f, line)) {
-        if (line.find(want) == std::string::npos) continue;
-        sepconv_choice_t b[3];
-        if (parse_choice(line, "2d", &b[0]) && parse_choice(line, "sep", &b[1]) && parse_choice(line, "auto", &b[2])) {
-            std::memcpy(best, b, sizeof b);
-            found = true;   // the last matching line wins
+    while (std::getline(f, line))
+        if (line.compare(0, want.size(), want) == 0) {
+            *out = line;
+            found = true;
         }
-    }
     return found;
+}
+
+bool load_choices(const std::string &path, const std::string &key, sepconv_choice_t best[3]) {
+    std::string line;
+    if (!find_line(path, key, &line)) return false;
+    sepconv_choice_t b[3];
+    if (!(parse_choice(line, "2d", &b[0]) && parse_choice(line, "sep", &b[1]) && parse_choice(line, "auto", &b[2])))
+        return false;
+    for (auto &c : b) c.source = SEPCONV_SRC_TUNED;
+    std::memcpy(best, b, sizeof b);
+    return true;
 }
 
 // Read-modify-write of the JSON-lines cache under an exclusive flock on "<path>.lock", through a
@@ -124,9 +163,10 @@ void store_cache(const std::string &path, const std::string &key, const std::str
     std::vector<std::string> keep;
     {
         std::ifstream f(path);
-        std::string line, want = "\"key\":\"" + key + "\"";
+        std::string line;
+        const std::string want = "{\"key\":\"" + key + "\",";
         while (f && std::getline(f, line))
-            if (!line.empty() && line.find(want) == std::string::npos) keep.push_back(line);
+            if (!line.empty() && line.compare(0, want.size(), want) != 0) keep.push_back(line);
     }
     std::ostringstream tn;
     tn << path << ".tmp." << ::getpid() << "." << std::hash<std::thread::id>{}(std::this_thread::get_id());
@@ -150,46 +190,331 @@ void store_choices(const std::string &path, const std::string &key, const sepcon
                                choice_json(best[1]) + ",\"auto\":" + choice_json(best[2]) + "}");
 }
 
-// The paper's selector picks a rule by input-size cutoffs (SELECT).  Here: a
-// plan of an untuned shape adopts the cached choice of the nearest tuned size (same GPU,
-// SM count, K and image count; sizes compared in log2 of the pixel count, within 2x).
-bool select_nearest(const std::string &path, sepconv_plan_t p, sepconv_choice_t best[3]) {
-    std::ifstream f(path);
-    if (!f) return false;
-    std::ostringstream pre;
-    pre << p->dev.name << "|" << p->dev.sms << "|";
-    const std::string want_pre = "\"key\":\"" + pre.str();
-    const double my = std::log2(static_cast<double>(p->h) * static_cast<double>(p->w));
-    double best_d = 1.0 + 1e-9;
-    bool found = false;
+void store_selector(const std::string &path, const std::string &key, const sepconv_selector_t &s) {
+    std::ostringstream o;
+    o << "{\"key\":\"" << key << "\",\"k\":" << s.k << ",\"m\":" << s.m << ",\"cutoffs\":[";
+    for (int i = 0; i + 1 < s.m; ++i) o << (i ? "," : "") << static_cast<long long>(s.cutoffs[i]);
+    o << "],\"algos\":[";
+    for (int i = 0; i < s.m; ++i) o << (i ? "," : "") << choice_json(s.algos[i]);
+    o << "]}";
+    store_cache(path, key, o.str());
+}
+
+bool load_selector(const std::string &path, const std::string &key, sepconv_selector_t *s) {
     std::string line;
-    while (std::getline(f, line)) {
-        const size_t at = line.find(want_pre);
-        if (at == std::string::npos) continue;
-        long long n = 0, h = 0, w = 0;
-        int k = 0;
-        if (sscanf(line.c_str() + at + want_pre.size(), "%lldx%lldx%lld|k%d", &n, &h, &w, &k) != 4) continue;
-        if (k != p->k || n != p->n) continue;
-        const double d = std::fabs(std::log2(static_cast<double>(h) * static_cast<double>(w)) - my);
-        sepconv_choice_t b[3];
-        if (d < best_d && parse_choice(line, "2d", &b[0]) && parse_choice(line, "sep", &b[1]) &&
-            parse_choice(line, "auto", &b[2])) {
-            best_d = d;
-            std::memcpy(best, b, sizeof b);
-            found = true;
+    if (!find_line(path, key, &line)) return false;
+    sepconv_selector_t r;
+    std::memset(&r, 0, sizeof r);
+    const size_t pk = line.find("\"k\":"), pm = line.find("\"m\":"), pc = line.find("\"cutoffs\":["),
+                 pa = line.find("\"algos\":[");
+    if (pk == std::string::npos || pm == std::string::npos || pc == std::string::npos || pa == std::string::npos)
+        return false;
+    if (sscanf(line.c_str() + pk + 4, "%d", &r.k) != 1 || sscanf(line.c_str() + pm + 4, "%d", &r.m) != 1) return false;
+    if (r.m < 1 || r.m > SEPCONV_SELECTOR_LEVELS) return false;
+    const char *p = line.c_str() + pc + 11;
+    for (int i = 0; i + 1 < r.m; ++i) {
+        long long v;
+        int used = 0;
+        if (sscanf(p, i ? ",%lld%n" : "%lld%n", &v, &used) != 1 || used == 0) return false;
+        r.cutoffs[i] = v;
+        p += used;
+    }
+    p = line.c_str() + pa + 9;
+    for (int i = 0; i < r.m; ++i) {
+        if (i) {
+            if (*p != ',') return false;
+            ++p;
+        }
+        p = parse_choice_at(p, &r.algos[i]);
+        if (!p) return false;
+        r.algos[i].source = SEPCONV_SRC_SELECTOR;
+    }
+    *s = r;
+    return true;
+}
+
+std::string cache_path_of(const sepconv_tune_opts_t *opts) {
+    if (opts && opts->cache_path) return opts->cache_path;
+    if (const char *env = std::getenv("SEPCONV_TUNE_CACHE")) return env;
+    return std::string();
+}
+
+// ---- timing -----------------------------------------------------------------------------------
+// Synthetic buffers and the flush machinery of one tuning session on one plan.
+struct Bench {
+    sepconv_plan_t plan = nullptr;
+    Geometry g{};
+    float *din = nullptr, *dout = nullptr, *wflush = nullptr, *rflush = nullptr, *sink = nullptr;
+    size_t flush_floats = 0;
+    bool need_flush = false;
+    cudaStream_t st = nullptr;
+    cudaEvent_t e0 = nullptr, e1 = nullptr;
+    std::vector<float> kern;
+
+    sepconv_status_t open(sepconv_plan_t p, bool allow_flush) {
+        plan = p;
+        const size_t in_floats = static_cast<size_t>(p->n * p->h * p->ld_in);
+        const size_t out_floats = static_cast<size_t>(p->n * p->ho * p->ld_out);
+        flush_floats = p->dev.l2 / 2;                     // 2 x L2 bytes
+        need_flush = allow_flush && (in_floats + out_floats) * 4 < 2 * p->dev.l2;
+        cudaError_t e;
+        if ((e = cudaMalloc(&din, in_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(in)");
+        if ((e = cudaMalloc(&dout, out_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(out)");
+        if (need_flush) {
+            if ((e = cudaMalloc(&wflush, flush_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(flush)");
+            if ((e = cudaMalloc(&rflush, flush_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(flush)");
+            if ((e = cudaMalloc(&sink, 16)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(sink)");
+        }
+        if ((e = cudaStreamCreateWithFlags(&st, cudaStreamNonBlocking)) != cudaSuccess) return cuda_fail(e, "tune: stream");
+        if ((e = cudaEventCreate(&e0)) != cudaSuccess || (e = cudaEventCreate(&e1)) != cudaSuccess)
+            return cuda_fail(e, "tune: events");
+        if (need_flush && (e = cudaMemsetAsync(rflush, 0, flush_floats * 4, st)) != cudaSuccess)
+            return cuda_fail(e, "tune: memset");
+        launch_fill_pattern(din, static_cast<long long>(in_floats), 1234u, st);
+        g = plan_geometry(p);
+        kern.resize(p->k);
+        for (int i = 0; i < p->k; ++i) {   // normalised binomial (the benchmark kernel)
+            double c = 1;
+            for (int j = 0; j < i; ++j) c = c * (p->k - 1 - j) / (j + 1);
+            kern[i] = static_cast<float>(c / std::pow(2.0, p->k - 1));
+        }
+        return SEPCONV_OK;
+    }
+    ~Bench() {
+        if (st) cudaStreamSynchronize(st);
+        for (float *b : {din, dout, wflush, rflush, sink})
+            if (b) cudaFree(b);
+        if (e0) cudaEventDestroy(e0);
+        if (e1) cudaEventDestroy(e1);
+        if (st) cudaStreamDestroy(st);
+    }
+    void flush() {
+        launch_l2_flush(wflush, static_cast<long long>(flush_floats), st);
+        launch_l2_clean(rflush, static_cast<long long>(flush_floats), sink, st);
+    }
+    // event time of n iterations of body, in us per iteration
+    sepconv_status_t batch(int n, const std::function<sepconv_status_t()> &body, double *us) {
+        cudaEventRecord(e0, st);
+        for (int i = 0; i < n; ++i) {
+            sepconv_status_t s = body();
+            if (s != SEPCONV_OK) return s;
+        }
+        cudaEventRecord(e1, st);
+        cudaError_t e = cudaEventSynchronize(e1);
+        if (e != cudaSuccess) return cuda_fail(e, "tune: run");
+        float ms = 0.f;
+        cudaEventElapsedTime(&ms, e0, e1);
+        *us = ms * 1000.0 / n;
+        return SEPCONV_OK;
+    }
+    // the pass time of candidate c: median of three batches of n (see the file comment)
+    sepconv_status_t time(const Candidate &c, int n, float *out_us) {
+        if (c.algo == SEPCONV_SEPARABLE && !c.fused) {
+            sepconv_status_t s = ensure_buf(plan);
+            if (s != SEPCONV_OK) return s;
+        }
+        auto pass = [&]() { return launch_candidate(plan, g, din, dout, kern.data(), c, plan->buf, plan->ld_buf, st); };
+        auto fl = [&]() {
+            flush();
+            return SEPCONV_OK;
+        };
+        auto flpass = [&]() {
+            flush();
+            return pass();
+        };
+        sepconv_status_t s = pass();                              // warm-up (first-launch costs)
+        if (s != SEPCONV_OK) return s;
+        double t[3];
+        for (int b = 0; b < 3; ++b) {
+            if (need_flush) {
+                double tf = 0, tfp = 0;
+                if ((s = batch(n, fl, &tf)) != SEPCONV_OK || (s = batch(n, flpass, &tfp)) != SEPCONV_OK) return s;
+                t[b] = std::max(0.05, tfp - tf);
+            } else {
+                if ((s = batch(n, pass, &t[b])) != SEPCONV_OK) return s;
+            }
+        }
+        std::sort(t, t + 3);
+        *out_us = static_cast<float>(t[1]);
+        return SEPCONV_OK;
+    }
+};
+
+// splitmix64 stream for the mutation search (reproducible for a given seed)
+struct Rng {
+    uint64_t s;
+    uint64_t next() {
+        uint64_t z = (s += 0x9E3779B97F4A7C15ull);
+        z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+        z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+        return z ^ (z >> 31);
+    }
+    double uniform() { return ((next() >> 11) + 0.5) * (1.0 / 9007199254740992.0); }
+    double normal() { return std::sqrt(-2.0 * std::log(uniform())) * std::cos(6.283185307179586 * uniform()); }
+};
+
+// Mutation search over the winner's work schedule.  The parent starts as the
+// model's schedule written as an explicit (parts, grid); each child scales one or both by
+// exp(sigma N(0,1)), sigma = ln 2 / 2 (a doubling or a halving is a 2-sigma step), and replaces
+// the parent only if it is faster by more than 1% (beyond timing noise; R23).
+sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int mutations, uint32_t seed, int reps) {
+    if (mutations <= 0 || passes(best) != 1) return SEPCONV_OK;
+    Sched model;
+    long long slots = 0;
+    Candidate probe = best;
+    probe.sched_parts = probe.sched_grid = 0;
+    sepconv_status_t s = candidate_sched(b.plan, b.g, probe, &model, &slots);
+    if (s != SEPCONV_OK) return s;
+    const int rows = b.g.rows;
+    const int cta_cols = candidate_warps(b.g.K, best) * kWarpCols;
+    const long long strips = static_cast<long long>(b.g.nimg) * ((b.g.out_cols + cta_cols - 1) / cta_cols);
+    double parts = model.parts > 0 ? model.parts
+                                   : std::max(1.0, std::round(static_cast<double>(slots) / std::max(1LL, strips)));
+    double grid = std::min(static_cast<double>(slots), static_cast<double>(strips) * parts);
+    Rng rng{0x5EC0A11Dull ^ (static_cast<uint64_t>(seed ? seed : 1u) << 17) ^ static_cast<uint64_t>(rows) ^
+            (static_cast<uint64_t>(b.g.K) << 40)};
+    const double sigma = 0.5 * std::log(2.0);
+    Candidate parent = best;
+    float parent_us = best_us;
+    for (int m = 0; m < mutations; ++m) {
+        const double u = rng.uniform();
+        double np = parts, ng = grid;
+        if (u < 2.0 / 3.0) np = parts * std::exp(sigma * rng.normal());
+        if (u >= 1.0 / 3.0) ng = grid * std::exp(sigma * rng.normal());
+        np = std::min<double>(std::max(1.0, std::round(np)), rows);
+        ng = std::min(std::max(1.0, std::round(ng)), static_cast<double>(slots));
+        Candidate child = parent;
+        child.sched_parts = static_cast<int>(np);
+        child.sched_grid = static_cast<int>(ng);
+        float us = 0.f;
+        if ((s = b.time(child, reps, &us)) != SEPCONV_OK) return s;
+        if (us < parent_us * 0.99f) {
+            parent = child;
+            parent_us = us;
+            parts = np;
+            grid = ng;
         }
     }
-    return found;
+    best = parent;
+    best_us = parent_us;
+    return SEPCONV_OK;
+}
+
+struct DeviceRestore {
+    int prev = -1;
+    explicit DeviceRestore(int dev) {
+        cudaGetDevice(&prev);
+        cudaSetDevice(dev);
+    }
+    ~DeviceRestore() {
+        if (prev >= 0) cudaSetDevice(prev);
+    }
+};
+
+// The exhaustive pass (+ mutation) on plan; fills best[3] (2D, SEPARABLE, AUTO).
+sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutations, uint32_t seed,
+                           sepconv_choice_t best[3]) {
+    DeviceRestore restore(plan->dev.device);
+    sepconv_status_t status;
+    auto cs = candidates(plan);
+    std::vector<float> med(cs.size(), -1.f);
+    Bench b;
+    if ((status = b.open(plan, !(flags & SEPCONV_TUNE_NO_L2_FLUSH))) != SEPCONV_OK) return status;
+    for (size_t ci = 0; ci < cs.size(); ++ci)
+        if ((status = b.time(cs[ci], reps, &med[ci])) != SEPCONV_OK) return status;
+
+    auto better = [&](size_t a, size_t c) {   // is candidate a better than incumbent c?
+        if (med[a] < 0) return false;
+        if (med[c] < 0) return true;
+        if (med[a] < med[c] * 0.99f) return true;
+        if (med[c] < med[a] * 0.99f) return false;
+        if (passes(cs[a]) != passes(cs[c])) return passes(cs[a]) < passes(cs[c]);
+        return false;   // keep the lower index
+    };
+    size_t bi[3] = {SIZE_MAX, SIZE_MAX, SIZE_MAX};
+    for (size_t i = 0; i < cs.size(); ++i) {
+        const int slot = cs[i].algo == SEPCONV_2D ? 0 : 1;
+        if (bi[slot] == SIZE_MAX || better(i, bi[slot])) bi[slot] = i;
+        if (bi[2] == SIZE_MAX || better(i, bi[2])) bi[2] = i;
+    }
+    Candidate win[3];
+    float us[3];
+    for (int s = 0; s < 3; ++s) {
+        win[s] = cs[bi[s]];
+        us[s] = med[bi[s]];
+    }
+    // the paper's evolutionary refinement of size-like tunables, on AUTO's winner
+    if ((status = mutate_schedule(b, win[2], us[2], mutations, seed, reps)) != SEPCONV_OK) return status;
+    const int aslot = win[2].algo == SEPCONV_2D ? 0 : 1;
+    if (bi[aslot] == bi[2]) {
+        win[aslot] = win[2];
+        us[aslot] = us[2];
+    }
+    for (int s = 0; s < 3; ++s) {
+        best[s] = to_choice(win[s], plan->k, SEPCONV_SRC_TUNED);
+        best[s].median_us = us[s];
+    }
+    return SEPCONV_OK;
+}
+
+int mutations_of(const sepconv_tune_opts_t *opts) {
+    if (!opts || opts->mutations == 0) return 12;
+    return opts->mutations < 0 ? 0 : opts->mutations;
+}
+
+sepconv_status_t square_plan(int64_t side, int K, int device, sepconv_plan_t *p) {
+    sepconv_plan_desc_t d;
+    std::memset(&d, 0, sizeof d);
+    d.n = 1;
+    d.h = d.w = side;
+    d.k = K;
+    d.device = device;
+    return sepconv_plan_ex(&d, p);
+}
+
+struct PlanHolder {
+    sepconv_plan_t p = nullptr;
+    ~PlanHolder() { sepconv_destroy(p); }
+};
+
+// times two choices on one plan (the cutoff placement of sepconv_tune_selector)
+sepconv_status_t time_pair(sepconv_plan_t p, const sepconv_choice_t &a, const sepconv_choice_t &c, int reps,
+                           int flags, float *ta, float *tc) {
+    DeviceRestore restore(p->dev.device);
+    Bench b;
+    sepconv_status_t s = b.open(p, !(flags & SEPCONV_TUNE_NO_L2_FLUSH));
+    if (s == SEPCONV_OK) s = b.time(from_choice(a), reps, ta);
+    if (s == SEPCONV_OK) s = b.time(from_choice(c), reps, tc);
+    return s;
 }
 
 }  // namespace
 
-// Called by sepconv_plan_ex: an exact cache hit makes the plan tuned; otherwise the nearest
-// tuned size class (NEXT-2 of SURVEY 8(f)) seeds AUTO / 2D / SEPARABLE until sepconv_tune.
+// Called by sepconv_plan_ex: an exact cache entry makes the plan tuned; otherwise a size
+// selector for its K (NEXT-2 of SURVEY 8(f)) resolves AUTO by SELECT until sepconv_tune.
 void sepconv_seed_from_cache(sepconv_plan_t plan) {
     const char *env = std::getenv("SEPCONV_TUNE_CACHE");
     if (!env || !*env) return;
-    if (load_cache(env, cache_key(plan), plan->best) || select_nearest(env, plan, plan->best)) plan->tuned = true;
+    if (load_choices(env, plan_key(plan), plan->best)) {
+        plan->tuned = true;
+        return;
+    }
+    sepconv_selector_t sel;
+    if (!load_selector(env, selector_key(plan->dev, plan->k), &sel) || sel.k != plan->k) return;
+    sepconv_choice_t pick;
+    if (sepconv_select(&sel, plan->n * plan->h * plan->w, &pick) != SEPCONV_OK) return;
+    pick.sched_parts = pick.sched_grid = 0;                    // size-specific: not transferred
+    const int slot = pick.algo == SEPCONV_2D ? 0 : 1;
+    for (int s = 0; s < 3; ++s) {
+        // 2D / SEPARABLE requests keep their static defaults unless the selector picked that algorithm
+        if (s == 2 || s == slot) {
+            plan->best[s] = pick;
+        } else {
+            Candidate d = resolve(plan, s == 0 ? SEPCONV_2D : SEPCONV_SEPARABLE);   // plan->tuned still false
+            plan->best[s] = to_choice(d, plan->k, SEPCONV_SRC_DEFAULT);
+        }
+    }
+    plan->tuned = true;
 }
 
 extern "C" {
@@ -203,14 +528,7 @@ sepconv_status_t sepconv_get_candidate(sepconv_plan_t plan, int index, sepconv_c
     if (!plan || !choice) return fail(SEPCONV_E_INVALID, "NULL argument");
     auto cs = candidates(plan);
     if (index < 0 || index >= static_cast<int>(cs.size())) return fail(SEPCONV_E_INVALID, "candidate index out of range");
-    std::memset(choice, 0, sizeof *choice);
-    choice->algo = static_cast<sepconv_variant_t>(cs[index].algo);
-    choice->mapping = cs[index].mapping;
-    choice->fused = cs[index].fused;
-    choice->config = cs[index].config;
-    choice->store_path = cs[index].store;
-    choice->warps = candidate_warps(plan->k, cs[index]);
-    choice->ctas_per_sm = 1;
+    *choice = to_choice(cs[index], plan->k, SEPCONV_SRC_EXPLICIT);
     return SEPCONV_OK;
 }
 
@@ -218,121 +536,102 @@ sepconv_status_t sepconv_tune(sepconv_plan_t plan, const sepconv_tune_opts_t *op
     if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
     const int reps = (opts && opts->reps > 0) ? opts->reps : 20;
     const int flags = opts ? opts->flags : 0;
-    std::string path;
-    if (opts && opts->cache_path) path = opts->cache_path;
-    else if (const char *env = std::getenv("SEPCONV_TUNE_CACHE")) path = env;
-    const std::string key = cache_key(plan);
+    const std::string path = cache_path_of(opts);
+    const std::string key = plan_key(plan);
 
-    if (!path.empty() && !(flags & SEPCONV_TUNE_FORCE) && load_cache(path, key, plan->best)) {
+    if (!path.empty() && !(flags & SEPCONV_TUNE_FORCE) && load_choices(path, key, plan->best)) {
         plan->tuned = true;
         if (chosen) *chosen = plan->best[2];
         return SEPCONV_OK;
     }
-
-    int prev = -1;
-    cudaGetDevice(&prev);
-    cudaSetDevice(plan->dev.device);
-    struct Restore {
-        int d;
-        ~Restore() {
-            if (d >= 0) cudaSetDevice(d);
-        }
-    } restore{prev};
-
-    const size_t in_floats = static_cast<size_t>(plan->n * plan->h * plan->ld_in);
-    const size_t out_floats = static_cast<size_t>(plan->n * plan->ho * plan->ld_out);
-    float *din = nullptr, *dout = nullptr, *flush = nullptr;
-    cudaStream_t st = nullptr;
-    cudaEvent_t e0 = nullptr, e1 = nullptr;
-    sepconv_status_t status = SEPCONV_OK;
-    const size_t flush_floats = plan->dev.l2 / 2;   // 2x L2 bytes
-    const bool need_flush = !(flags & SEPCONV_TUNE_NO_L2_FLUSH) &&
-                            (in_floats + out_floats) * 4 < 2 * plan->dev.l2;
-    std::vector<float> kern(plan->k);
-    for (int i = 0; i < plan->k; ++i) {   // normalised binomial (the benchmark kernel)
-        double c = 1;
-        for (int j = 0; j < i; ++j) c = c * (plan->k - 1 - j) / (j + 1);
-        kern[i] = static_cast<float>(c / std::pow(2.0, plan->k - 1));
-    }
-    auto cs = candidates(plan);
-    std::vector<float> med(cs.size(), -1.f);
-
-    do {
-        cudaError_t e;
-        if ((e = cudaMalloc(&din, in_floats * 4)) != cudaSuccess) { status = cuda_fail(e, "tune: cudaMalloc(in)"); break; }
-        if ((e = cudaMalloc(&dout, out_floats * 4)) != cudaSuccess) { status = cuda_fail(e, "tune: cudaMalloc(out)"); break; }
-        if (need_flush && (e = cudaMalloc(&flush, flush_floats * 4)) != cudaSuccess) {
-            status = cuda_fail(e, "tune: cudaMalloc(flush)");
-            break;
-        }
-        if ((e = cudaStreamCreateWithFlags(&st, cudaStreamNonBlocking)) != cudaSuccess) { status = cuda_fail(e, "tune: stream"); break; }
-        cudaEventCreate(&e0);
-        cudaEventCreate(&e1);
-        launch_fill_pattern(din, static_cast<long long>(in_floats), 1234u, st);
-        Geometry g = plan_geometry(plan);
-        for (size_t ci = 0; ci < cs.size() && status == SEPCONV_OK; ++ci) {
-            const Candidate &c = cs[ci];
-            if (c.algo == SEPCONV_SEPARABLE && !c.fused) {
-                status = ensure_buf(plan);
-                if (status != SEPCONV_OK) break;
-            }
-            std::vector<float> t;
-            for (int r = 0; r < reps + 2; ++r) {
-                if (need_flush) launch_l2_flush(flush, static_cast<long long>(flush_floats), st);
-                cudaEventRecord(e0, st);
-                status = launch_candidate(plan, g, din, dout, kern.data(), c, plan->buf, plan->ld_buf, st);
-                if (status != SEPCONV_OK) break;
-                cudaEventRecord(e1, st);
-                if ((e = cudaEventSynchronize(e1)) != cudaSuccess) { status = cuda_fail(e, "tune: run"); break; }
-                float ms = 0;
-                cudaEventElapsedTime(&ms, e0, e1);
-                if (r >= 2) t.push_back(ms * 1000.f);
-            }
-            if (status != SEPCONV_OK) break;
-            std::sort(t.begin(), t.end());
-            med[ci] = t[t.size() / 2];
-        }
-    } while (0);
-
-    if (st) cudaStreamSynchronize(st);
-    if (din) cudaFree(din);
-    if (dout) cudaFree(dout);
-    if (flush) cudaFree(flush);
-    if (e0) cudaEventDestroy(e0);
-    if (e1) cudaEventDestroy(e1);
-    if (st) cudaStreamDestroy(st);
-    if (status != SEPCONV_OK) return status;
-
-    auto better = [&](size_t a, size_t b) {   // is candidate a better than incumbent b?
-        if (med[a] < 0) return false;
-        if (med[b] < 0) return true;
-        if (med[a] < med[b] * 0.99f) return true;
-        if (med[b] < med[a] * 0.99f) return false;
-        if (passes(cs[a]) != passes(cs[b])) return passes(cs[a]) < passes(cs[b]);
-        return false;   // keep the lower index
-    };
-    size_t bi[3] = {SIZE_MAX, SIZE_MAX, SIZE_MAX};
-    for (size_t i = 0; i < cs.size(); ++i) {
-        const int slot = cs[i].algo == SEPCONV_2D ? 0 : 1;
-        if (bi[slot] == SIZE_MAX || better(i, bi[slot])) bi[slot] = i;
-        if (bi[2] == SIZE_MAX || better(i, bi[2])) bi[2] = i;
-    }
-    for (int s = 0; s < 3; ++s) {
-        const Candidate &c = cs[bi[s]];
-        sepconv_choice_t &o = plan->best[s];
-        std::memset(&o, 0, sizeof o);
-        o.algo = static_cast<sepconv_variant_t>(c.algo);
-        o.mapping = c.mapping;
-        o.fused = c.fused;
-        o.config = c.config;
-        o.store_path = c.store;
-        o.warps = candidate_warps(plan->k, c);
-        o.ctas_per_sm = 1;
-        o.median_us = med[bi[s]];
-    }
+    sepconv_choice_t best[3];
+    sepconv_status_t s = tune_plan(plan, reps, flags, mutations_of(opts), opts ? opts->seed : 0u, best);
+    if (s != SEPCONV_OK) return s;
+    std::memcpy(plan->best, best, sizeof best);
     plan->tuned = true;
     if (!path.empty()) store_choices(path, key, plan->best);
     if (chosen) *chosen = plan->best[2];
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_select(const sepconv_selector_t *s, int64_t size, sepconv_choice_t *choice) {
+    if (!s || !choice) return fail(SEPCONV_E_INVALID, "NULL argument");
+    if (s->m < 1 || s->m > SEPCONV_SELECTOR_LEVELS) return fail(SEPCONV_E_INVALID, "selector m=%d outside 1..12", s->m);
+    if (s->m > 1 && s->cutoffs[0] <= 0) return fail(SEPCONV_E_INVALID, "selector cutoff c_1 must be > 0");
+    for (int i = 1; i + 1 < s->m; ++i)
+        if (!(s->cutoffs[i] > s->cutoffs[i - 1])) return fail(SEPCONV_E_INVALID, "selector cutoffs not increasing");
+    // alpha_i such that c_i > size >= c_{i-1}, c_0 = 0, c_m = infinity
+    int i = 0;
+    while (i + 1 < s->m && size >= s->cutoffs[i]) ++i;
+    *choice = s->algos[i];
+    choice->source = SEPCONV_SRC_SELECTOR;
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_tune_selector(int K, int device, const int64_t *sides, int nsides,
+                                       const sepconv_tune_opts_t *opts, sepconv_selector_t *out) {
+    static const int64_t kLevels[SEPCONV_SELECTOR_LEVELS] = {64, 128, 256, 512, 1024, 2048,
+                                                             3072, 4096, 6144, 8192, 11584, 16384};
+    if (K < 1 || K > SEPCONV_MAX_K) return fail(SEPCONV_E_UNSUPPORTED, "K=%d outside 1..%d", K, SEPCONV_MAX_K);
+    if (!sides) {
+        sides = kLevels;
+        nsides = SEPCONV_SELECTOR_LEVELS;
+    }
+    if (nsides < 1 || nsides > SEPCONV_SELECTOR_LEVELS) return fail(SEPCONV_E_INVALID, "nsides must be in 1..12");
+    for (int i = 0; i < nsides; ++i)
+        if (sides[i] < K || (i && sides[i] <= sides[i - 1]))
+            return fail(SEPCONV_E_INVALID, "sides must be >= K and strictly increasing");
+    const int reps = (opts && opts->reps > 0) ? opts->reps : 10;
+    const int flags = opts ? opts->flags : 0;
+    auto same = [](const sepconv_choice_t &a, const sepconv_choice_t &c) {
+        return std::make_tuple(static_cast<int>(a.algo), a.mapping, a.fused, a.config, a.store_path) ==
+               std::make_tuple(static_cast<int>(c.algo), c.mapping, c.fused, c.config, c.store_path);
+    };
+    // 1. the exhaustive tuner (no mutation: schedules are size-specific) at every level
+    std::vector<sepconv_choice_t> pick(nsides);
+    DeviceInfo dev;
+    for (int i = 0; i < nsides; ++i) {
+        PlanHolder h;
+        sepconv_status_t s = square_plan(sides[i], K, device, &h.p);
+        if (s != SEPCONV_OK) return s;
+        dev = h.p->dev;
+        sepconv_choice_t best[3];
+        if ((s = tune_plan(h.p, reps, flags, 0, 0u, best)) != SEPCONV_OK) return s;
+        pick[i] = best[2];
+    }
+    // 2. merge equal neighbours; 3. place each cutoff between two different picks by timing
+    // both at the geometric middle side of the two levels (one bisection step in log size)
+    sepconv_selector_t sel;
+    std::memset(&sel, 0, sizeof sel);
+    sel.k = K;
+    sel.m = 1;
+    sel.algos[0] = pick[0];
+    for (int i = 1; i < nsides; ++i) {
+        if (same(pick[i], sel.algos[sel.m - 1])) continue;
+        const double lo = static_cast<double>(sides[i - 1]), hi = static_cast<double>(sides[i]);
+        const int64_t mid = std::llround(std::sqrt(lo * hi));
+        int64_t cut_side = mid;                               // the side where pick[i] takes over
+        if (mid > sides[i - 1] && mid < sides[i]) {
+            PlanHolder h;
+            sepconv_status_t s = square_plan(mid, K, device, &h.p);
+            float t_lo = 0.f, t_hi = 0.f;
+            if (s == SEPCONV_OK) s = time_pair(h.p, sel.algos[sel.m - 1], pick[i], reps, flags, &t_lo, &t_hi);
+            if (s != SEPCONV_OK) return s;
+            // the lower level's pick still wins at the middle: the switch lies above it
+            cut_side = t_lo <= t_hi ? std::llround(std::sqrt(static_cast<double>(mid) * hi))
+                                    : std::llround(std::sqrt(lo * static_cast<double>(mid)));
+        }
+        sel.cutoffs[sel.m - 1] = cut_side * cut_side;         // size = n*h*w pixels
+        sel.algos[sel.m] = pick[i];
+        ++sel.m;
+    }
+    for (int i = 0; i < sel.m; ++i) {
+        sel.algos[i].sched_parts = sel.algos[i].sched_grid = 0;
+        sel.algos[i].source = SEPCONV_SRC_SELECTOR;
+    }
+    const std::string path = cache_path_of(opts);
+    if (!path.empty()) store_selector(path, selector_key(dev, K), sel);
+    if (out) *out = sel;
     return SEPCONV_OK;
 }
 

@@ -19,7 +19,25 @@ __global__ void l2_flush_kernel(float4 *dst, long long n4) {
     for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n4; i += (long long)gridDim.x * blockDim.x)
         dst[i] = v;
 }
+// Reads a buffer larger than L2 after the write flush, so the lines left in L2 are clean: a
+// timed pass then pays only for its own traffic, not for writing back ~L2-size of dirty lines
+// that an unrelated kernel left behind (profiles/r02_flush_study.txt).  The sum is stored only
+// if it is negative, which never happens for the non-negative contents, but the compiler
+// cannot drop the loads.
+__global__ void l2_clean_kernel(const float4 *__restrict__ src, long long n4, float *sink) {
+    float acc = 0.f;
+    for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n4; i += (long long)gridDim.x * blockDim.x) {
+        const float4 v = src[i];                     // normal allocation (not evict-first)
+        acc += (v.x + v.y) + (v.z + v.w);
+    }
+    if (acc < 0.f) *sink = acc;
+}
 }  // namespace
+
+cudaError_t launch_l2_clean(const float *src, long long n, float *sink, cudaStream_t st) {
+    l2_clean_kernel<<<148 * 8, 256, 0, st>>>(reinterpret_cast<const float4 *>(src), n / 4, sink);
+    return cudaGetLastError();
+}
 
 cudaError_t launch_fill_pattern(float *dst, long long n, unsigned seed, cudaStream_t st) {
     fill_pattern_kernel<<<148 * 8, 256, 0, st>>>(dst, n, seed);

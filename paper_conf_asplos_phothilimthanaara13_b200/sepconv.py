@@ -23,6 +23,8 @@ LIB_PATH = os.path.join(_HERE, "libsepconv.so")
 SEPCONV_2D, SEPCONV_SEPARABLE, SEPCONV_AUTO = 0, 1, 2
 MAP_DIRECT, MAP_TMA = 0, 1
 TUNE_FORCE, TUNE_NO_L2_FLUSH = 1, 2
+SRC_DEFAULT, SRC_TUNED, SRC_SELECTOR, SRC_EXPLICIT = 0, 1, 2, 3
+SELECTOR_LEVELS = 12
 MAX_K = 17
 NCCL_ID_BYTES = 128
 VARIANTS = {"2d": SEPCONV_2D, "separable": SEPCONV_SEPARABLE, "auto": SEPCONV_AUTO}
@@ -47,11 +49,18 @@ class _Choice(ctypes.Structure):
     _fields_ = [("algo", ctypes.c_int), ("mapping", ctypes.c_int), ("fused", ctypes.c_int),
                 ("config", ctypes.c_int), ("store_path", ctypes.c_int), ("warps", ctypes.c_int),
                 ("ctas_per_sm", ctypes.c_int),
-                ("median_us", ctypes.c_float)]
+                ("median_us", ctypes.c_float), ("sched_parts", ctypes.c_int), ("sched_grid", ctypes.c_int),
+                ("source", ctypes.c_int)]
 
 
 class _TuneOpts(ctypes.Structure):
-    _fields_ = [("reps", ctypes.c_int), ("cache_path", ctypes.c_char_p), ("flags", ctypes.c_int)]
+    _fields_ = [("reps", ctypes.c_int), ("cache_path", ctypes.c_char_p), ("flags", ctypes.c_int),
+                ("mutations", ctypes.c_int), ("seed", ctypes.c_uint32)]
+
+
+class _Selector(ctypes.Structure):
+    _fields_ = [("k", ctypes.c_int), ("m", ctypes.c_int), ("cutoffs", ctypes.c_int64 * (SELECTOR_LEVELS - 1)),
+                ("algos", _Choice * SELECTOR_LEVELS)]
 
 
 @dataclass(frozen=True)
@@ -64,25 +73,64 @@ class Choice:
     warps: int = 8
     ctas_per_sm: int = 1
     median_us: float = 0.0
+    sched_parts: int = 0          # tuned work-schedule override (0 = the library's model)
+    sched_grid: int = 0
+    source: int = SRC_EXPLICIT    # SRC_DEFAULT / SRC_TUNED / SRC_SELECTOR / SRC_EXPLICIT
 
     @property
-    def name(self) -> str:
+    def base_name(self) -> str:
+        """The candidate's name without a schedule override."""
         a = "2d" if self.algo == SEPCONV_2D else ("sep-fused" if self.fused else "sep-unfused")
         m = ("-tma" if self.mapping == MAP_TMA else "-direct")
         if self.algo == SEPCONV_SEPARABLE and self.fused and self.mapping == MAP_TMA:
             m += "%d" % self.config + ("s8" if self.store_path else "")
         return a + m
 
+    @property
+    def name(self) -> str:
+        return self.base_name + ("@p%dg%d" % (self.sched_parts, self.sched_grid) if self.sched_parts else "")
+
     def key(self):
-        return (self.algo, self.mapping, self.fused, self.config, self.store_path)
+        return (self.algo, self.mapping, self.fused, self.config, self.store_path, self.sched_parts, self.sched_grid)
 
     def _c(self) -> _Choice:
         return _Choice(self.algo, self.mapping, self.fused, self.config, self.store_path, self.warps, self.ctas_per_sm,
-                       self.median_us)
+                       self.median_us, self.sched_parts, self.sched_grid, self.source)
 
     @staticmethod
     def _from(c: _Choice) -> "Choice":
-        return Choice(c.algo, c.mapping, c.fused, c.config, c.store_path, c.warps, c.ctas_per_sm, float(c.median_us))
+        return Choice(c.algo, c.mapping, c.fused, c.config, c.store_path, c.warps, c.ctas_per_sm, float(c.median_us),
+                      c.sched_parts, c.sched_grid, c.source)
+
+
+@dataclass(frozen=True)
+class Selector:
+    """sepconv_selector_t: SELECT(input, s) = algos[i] with cutoffs[i] > n*h*w >= cutoffs[i-1]
+    (P:820-829)."""
+    k: int
+    cutoffs: tuple
+    algos: tuple
+
+    def _c(self) -> _Selector:
+        s = _Selector()
+        s.k, s.m = self.k, len(self.algos)
+        for i, c in enumerate(self.cutoffs):
+            s.cutoffs[i] = int(c)
+        for i, a in enumerate(self.algos):
+            s.algos[i] = a._c()
+        return s
+
+    @staticmethod
+    def _from(s: _Selector) -> "Selector":
+        return Selector(s.k, tuple(int(s.cutoffs[i]) for i in range(s.m - 1)),
+                        tuple(Choice._from(s.algos[i]) for i in range(s.m)))
+
+    def select(self, size: int) -> Choice:
+        """sepconv_select (host arithmetic in the library)."""
+        out = _Choice()
+        c = self._c()
+        _check(lib().sepconv_select(ctypes.byref(c), int(size), ctypes.byref(out)), "sepconv_select")
+        return Choice._from(out)
 
 
 _lib = None
@@ -110,6 +158,9 @@ def lib() -> ctypes.CDLL:
             "sepconv_run_choice": (I, [P, P, P, P, ctypes.POINTER(_Choice), P]),
             "sepconv_run_host": (I, [P, P, P, P, I, P]),
             "sepconv_tune": (I, [P, ctypes.POINTER(_TuneOpts), ctypes.POINTER(_Choice)]),
+            "sepconv_tune_selector": (I, [I, I, ctypes.POINTER(ctypes.c_int64), I, ctypes.POINTER(_TuneOpts),
+                                          ctypes.POINTER(_Selector)]),
+            "sepconv_select": (I, [ctypes.POINTER(_Selector), I64, ctypes.POINTER(_Choice)]),
             "sepconv_get_choice": (I, [P, I, ctypes.POINTER(_Choice)]),
             "sepconv_num_candidates": (I, [P]),
             "sepconv_get_candidate": (I, [P, I, ctypes.POINTER(_Choice)]),
@@ -147,7 +198,8 @@ def launch_count() -> int:
 
 def exported_symbols():
     return ["sepconv_plan", "sepconv_plan_ex", "sepconv_destroy", "sepconv_out_shape", "sepconv_run",
-            "sepconv_run_choice", "sepconv_run_host", "sepconv_tune", "sepconv_get_choice",
+            "sepconv_run_choice", "sepconv_run_host", "sepconv_tune", "sepconv_tune_selector", "sepconv_select",
+            "sepconv_get_choice",
             "sepconv_num_candidates", "sepconv_get_candidate", "sepconv_band", "sepconv_nccl_unique_id",
             "sepconv_comm_init", "sepconv_run_band", "sepconv_status_str", "sepconv_last_error",
             "sepconv_version", "sepconv_launch_count"]
@@ -266,9 +318,10 @@ class Plan:
 
     # -- tuning --
     def tune(self, reps: int = 20, cache_path: str | None = None, force: bool = False,
-             no_l2_flush: bool = False) -> Choice:
+             no_l2_flush: bool = False, mutations: int = 0, seed: int = 0) -> Choice:
+        """sepconv_tune: exhaustive pass + `mutations` schedule mutations (0 = 12, < 0 = none)."""
         flags = (TUNE_FORCE if force else 0) | (TUNE_NO_L2_FLUSH if no_l2_flush else 0)
-        opts = _TuneOpts(int(reps), cache_path.encode() if cache_path else None, flags)
+        opts = _TuneOpts(int(reps), cache_path.encode() if cache_path else None, flags, int(mutations), int(seed))
         out = _Choice()
         _check(lib().sepconv_tune(self._h, ctypes.byref(opts), ctypes.byref(out)), "sepconv_tune")
         return Choice._from(out)
@@ -298,6 +351,22 @@ class Plan:
         _check(lib().sepconv_run_band(self._h, _ptr(in_band), k.ctypes.data, _ptr(out_band), _variant(variant),
                                       _stream(stream)), "sepconv_run_band")
         return out_band
+
+
+def tune_selector(K: int, sides=None, reps: int = 10, cache_path: str | None = None, device: int = -1,
+                  no_l2_flush: bool = False) -> Selector:
+    """sepconv_tune_selector: the size selector for width K (12 square levels by default)."""
+    arr = None
+    n = 0
+    if sides is not None:
+        n = len(sides)
+        arr = (ctypes.c_int64 * n)(*[int(x) for x in sides])
+    opts = _TuneOpts(int(reps), cache_path.encode() if cache_path else None,
+                     TUNE_NO_L2_FLUSH if no_l2_flush else 0, -1, 0)
+    out = _Selector()
+    _check(lib().sepconv_tune_selector(int(K), int(device), arr, n, ctypes.byref(opts), ctypes.byref(out)),
+           "sepconv_tune_selector")
+    return Selector._from(out)
 
 
 def plan(H: int, W: int, K: int) -> Plan:

@@ -154,3 +154,35 @@ def test_sor_band_rejects_thin_bands_and_odd_halos():
         sor.band(40, 8, 0, 8)
     with pytest.raises(sc.SepconvError):
         sor.band(400, 2, 0, 3)
+
+
+# ---- the size selector's SELECT, pure host arithmetic --------------------------
+def _sel(cutoffs, n_algos):
+    algos = tuple(sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, i % 4) for i in range(n_algos))
+    return sc.Selector(7, tuple(cutoffs), algos)
+
+
+def test_select_follows_the_cutoff_definition():
+    """SELECT(input, s) = alpha_i s.t. c_i > size >= c_{i-1}, c_0 = 0, c_m = inf:
+    a size equal to a cutoff belongs to the level above it."""
+    s = _sel([1000, 50000], 3)
+    cases = {0: 0, 1: 0, 999: 0, 1000: 1, 1001: 1, 49999: 1, 50000: 2, 10 ** 12: 2}
+    for size, level in cases.items():
+        got = s.select(size)
+        assert got.config == level % 4, (size, got)
+        assert got.source == sc.SRC_SELECTOR
+    one = _sel([], 1)
+    assert one.select(0).config == 0 and one.select(2 ** 40).config == 0
+    full = _sel([4 ** i for i in range(1, 12)], 12)           # 12 levels: the paper's maximum
+    assert full.select(4 ** 11).config == 11 % 4 and full.select(4 ** 11 - 1).config == 10 % 4
+
+
+@pytest.mark.parametrize("cutoffs,m", [([500, 500], 3), ([900, 100], 3), ([0], 2), ([], 0)])
+def test_select_rejects_malformed_selectors(cutoffs, m):
+    s = sc._Selector()
+    s.k, s.m = 5, m
+    for i, c in enumerate(cutoffs):
+        s.cutoffs[i] = c
+    out = sc._Choice()
+    import ctypes
+    assert sc.lib().sepconv_select(ctypes.byref(s), 100, ctypes.byref(out)) == -1   # E_INVALID

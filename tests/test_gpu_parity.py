@@ -162,11 +162,11 @@ def test_tune_choice_is_valid_and_cached(tmp_path):
     best = p.tune(reps=3, cache_path=cache, force=True)
     assert best.median_us > 0
     names = {c.name for c in p.candidates()}
-    assert best.name in names
+    assert best.base_name in names and best.source == sc.SRC_TUNED
     for v in ("2d", "separable", "auto"):
         c = p.get_choice(v)
         assert c.median_us > 0
-        assert c.name in names
+        assert c.base_name in names
     # ties within 1% go to fewer passes / the lower candidate index (R17)
     assert p.get_choice("auto").median_us <= min(p.get_choice("2d").median_us, p.get_choice("separable").median_us) * 1.01
     check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
@@ -339,19 +339,60 @@ def test_run_band_nccl_single_rank_and_shared_comm():
     p2.close()
 
 
-def test_size_class_selector_seeds_untuned_plans(tmp_path, monkeypatch):
-    """NEXT-2: with $SEPCONV_TUNE_CACHE set, an untuned plan adopts the choice tuned for the
-    nearest image size (the paper's SELECT by input-size cutoffs)."""
+def test_size_selector_resolves_untuned_plans(tmp_path, monkeypatch):
+    """NEXT-2: sepconv_tune_selector builds SELECT's cutoff table for K over the 12 default
+    square levels and stores it in the tuning cache; a plan of an
+    untuned shape (3000^2, between the 2048 and 3072 levels) then resolves AUTO through it
+    (source SELECTOR, the same choice sepconv_select gives for 3000^2 pixels) and matches the
+    oracle on the whole output.  A shape with its own tuned entry still takes that entry."""
     cache = str(tmp_path / "tune.jsonl")
+    K = 9
+    sel = sc.tune_selector(K, reps=5, cache_path=cache)
+    assert 1 <= len(sel.algos) <= 12 and len(sel.cutoffs) == len(sel.algos) - 1
+    assert all(a < b for a, b in zip(sel.cutoffs, sel.cutoffs[1:]))
+    assert all(64 * 64 < c < 16384 * 16384 for c in sel.cutoffs)
     monkeypatch.setenv("SEPCONV_TUNE_CACHE", cache)
-    tuned = sc.Plan(1024, 1024, 9)
-    best = tuned.tune(reps=3, force=True)
-    near = sc.Plan(1100, 1000, 9)                          # 1.05x the pixels: same size class
-    assert near.get_choice("auto").key() == best.key()
-    far = sc.Plan(4096, 4096, 9)                           # 16x: not seeded
-    assert far.get_choice("auto").median_us == 0.0
-    img = synth.uniform_image(1100, 1000, seed=5)
-    check(img, synth.binomial_kernel(9), run_gpu(img, synth.binomial_kernel(9), variant="auto", plan=near)[0])
+    p = sc.Plan(3000, 3000, K)
+    got = p.get_choice("auto")
+    want = sel.select(3000 * 3000)
+    assert got.source == sc.SRC_SELECTOR and got.base_name == want.base_name, (got, want, sel)
+    img = synth.uniform_image(3000, 3000, seed=5)
+    k = synth.binomial_kernel(K)
+    check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
+    # an exact tuned entry wins over the selector
+    q = sc.Plan(512, 640, K)
+    q.tune(reps=3, cache_path=cache, force=True)
+    assert sc.Plan(512, 640, K).get_choice("auto").source == sc.SRC_TUNED
+
+
+def test_mutated_schedules_are_bitwise_equal_and_tuned_one_is_kept(tmp_path):
+    """Schedule overrides (the size-like tunables the mutation search scales) change
+    which CTA computes which rows, never a pixel's arithmetic (R6): every
+    (parts, grid) gives the model schedule's bits.  The tuner's mutated AUTO pick round-trips
+    through the cache and passes parity."""
+    h, w, K = 1500, 2300, 13
+    img = synth.uniform_image(h, w, seed=8)
+    k = synth.random_kernel(K, seed=3, signed=True)
+    p = sc.Plan(h, w, K)
+    dev = torch.from_numpy(img).cuda()
+    base = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2)
+    ref = torch.empty((h - K + 1, w - K + 1), device="cuda")
+    p.run_choice(dev, k, ref, base)
+    for parts, grid in ((1, 1), (1, 3), (7, 20), (40, 148), (3000, 148), (13, 0), (200, 37)):
+        out = torch.full_like(ref, float("nan"))
+        p.run_choice(dev, k, out, sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2, sched_parts=parts,
+                                            sched_grid=grid))
+        torch.cuda.synchronize()
+        assert torch.equal(out, ref), (parts, grid)
+    for c in (sc.Choice(sc.SEPCONV_2D, sc.MAP_TMA, 0, sched_parts=5, sched_grid=60),):
+        out = torch.full_like(ref, float("nan"))
+        p.run_choice(dev, k, out, c)
+        torch.cuda.synchronize()
+        check(img, k, out.cpu().numpy())
+    cache = str(tmp_path / "t.jsonl")
+    best = p.tune(reps=5, cache_path=cache, force=True, mutations=16, seed=7)
+    assert sc.Plan(h, w, K).tune(reps=5, cache_path=cache) == best
+    check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
 
 
 # ---- work schedules: the window schedule (every SM busy) equals the others bit for bit -----
