@@ -421,21 +421,33 @@ def main():
     if dist:
         dist.barrier()
 
-    # ---- timed region: CUDA events on the launching stream, per pass and per step ----
-    ev = {K: [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
-              for _ in range(args.steps)] for K in widths}
-    e_start, e_end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    # working sets that fit in L2 (in + out <= 2 x L2) are flushed before every pass, outside the
-    # per-pass events: a write of a 2 x L2 scratch buffer, then a read of a second 2 x L2 buffer so
-    # the pass starts from an L2 of clean, unrelated lines (a write alone leaves ~L2-size of dirty
-    # lines whose write-back the timed pass would pay: +2-6 us at 2048^2-4096^2,
-    # profiles/r02_flush_study.txt); ms_per_step is then the sum of the per-pass device times.
-    # Larger inputs stream from HBM anyway (no flush).
+    # ---- timed region: CUDA events on the launching stream ----
+    # Inputs larger than L2 (the default 16384^2, the batch) run the steps back to back: events
+    # around every pass and around the whole timed region.  Working sets that fit in L2 (in + out
+    # <= 2 x L2: 2048^2-4096^2) need a flush before every pass: a write of a 2 x L2 scratch buffer,
+    # then a read of a second 2 x L2 buffer, so the pass starts from an L2 of clean, unrelated
+    # lines (a write alone leaves ~L2-size of dirty lines whose write-back the pass would pay:
+    # +2-6 us, profiles/r02_flush_study.txt).  A single event pair around one short pass measures
+    # a ~5 us event/launch floor in 2.048 us ticks (profiles/r02_latency_probe.txt), so per
+    # width the flushed mode times `steps` x [flush, pass] and `steps` x [flush] between event
+    # pairs and takes the difference: the marginal device time of the pass inside a stream of
+    # work, as the unflushed mode measures it.
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
     scratch = torch.empty(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
     rscratch = torch.zeros(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
     sink = torch.empty((), dtype=torch.float32, device=dev)
+
+    def do_flush(s):
+        scratch.fill_(float(s))
+        torch.sum(rscratch, dim=0, out=sink)
+
+    def evpair():
+        return torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+
+    ev = {K: [evpair() for _ in range(args.steps)] for K in widths}
+    fev = {K: (evpair(), evpair()) for K in widths}
+    e_start, e_end = evpair()
     launches0 = sc.launch_count()
     with ClockSampler(local) as clk:
         torch.cuda.synchronize()
@@ -443,14 +455,24 @@ def main():
             dist.barrier()
         torch.cuda.nvtx.range_push("sepconv_timed")      # ncu --nvtx-include sepconv_timed/
         e_start.record(stream)
-        for s in range(args.steps):
+        if flush:
             for K in widths:
-                if flush:
-                    scratch.fill_(float(s))
-                    torch.sum(rscratch, dim=0, out=sink)
-                ev[K][s][0].record(stream)
-                one_pass(K)
-                ev[K][s][1].record(stream)
+                (a0, a1), (b0, b1) = fev[K]
+                a0.record(stream)
+                for s in range(args.steps):
+                    do_flush(s)
+                    one_pass(K)
+                a1.record(stream)
+                b0.record(stream)
+                for s in range(args.steps):
+                    do_flush(s)
+                b1.record(stream)
+        else:
+            for s in range(args.steps):
+                for K in widths:
+                    ev[K][s][0].record(stream)
+                    one_pass(K)
+                    ev[K][s][1].record(stream)
         e_end.record(stream)
         torch.cuda.nvtx.range_pop()
         torch.cuda.synchronize()
@@ -461,10 +483,13 @@ def main():
         tl = torch.tensor([launches], dtype=torch.int64, device=dev)
         dist.all_reduce(tl)
         launches = int(tl.item())
-    total_ms = e_start.elapsed_time(e_end)
-    per_k_ms = {K: sum(a.elapsed_time(b) for a, b in ev[K]) / args.steps for K in widths}
     if flush:                                    # the flushes are not part of the step
+        per_k_ms = {K: max(1e-6, fev[K][0][0].elapsed_time(fev[K][0][1]) - fev[K][1][0].elapsed_time(fev[K][1][1]))
+                    / args.steps for K in widths}
         total_ms = sum(per_k_ms.values()) * args.steps
+    else:
+        total_ms = e_start.elapsed_time(e_end)
+        per_k_ms = {K: sum(a.elapsed_time(b) for a, b in ev[K]) / args.steps for K in widths}
     if dist:
         t = torch.tensor([total_ms] + [per_k_ms[K] for K in widths], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
@@ -594,7 +619,8 @@ def main():
                "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
                "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
                "l2": ("L2 flushed before every pass (write 2 x L2, then read another 2 x L2 so L2 holds clean "
-                      "unrelated lines; outside the per-pass events; ms_per_step = sum of per-pass device times)")
+                      "unrelated lines); per width, pass time = [events around steps x (flush + pass)] - "
+                      "[events around steps x flush], / steps; ms_per_step = sum over widths")
                if flush else "inputs larger than L2 (no flush)",
                "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
                                else f"images sharded x{world}" if world > 1 else "1 GPU")}

@@ -503,7 +503,9 @@ sepconv_choice_t to_choice(const Candidate &c, int K, int source) {
     o.config = c.config;
     o.store_path = c.store;
     o.warps = candidate_warps(K, c);
-    o.ctas_per_sm = 1;
+    o.ctas_per_sm = (c.algo == SEPCONV_SEPARABLE && c.fused && c.mapping == SEPCONV_MAP_TMA)
+                        ? std::max(1, stream_info(OP_SEP, 2 + c.config, K, 1).cps)
+                        : 1;
     o.sched_parts = c.sched_parts;
     o.sched_grid = c.sched_grid;
     o.source = source;
@@ -684,10 +686,8 @@ static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const
     }
     Geometry g = plan_geometry(plan);
     // the unfused buffer for a whole-image launch is [n][h][ld_buf] (rows = ho + K - 1 = h)
-    s = launch_candidate(plan, g, in, out, kernel, c, plan->buf, plan->ld_buf, st);
-    if (s != SEPCONV_OK) return s;
-    cudaEventRecord(plan->last_work, st);
-    return SEPCONV_OK;
+    // (no per-call event: sepconv_destroy synchronises the device before freeing anything)
+    return launch_candidate(plan, g, in, out, kernel, c, plan->buf, plan->ld_buf, st);
 }
 
 sepconv_status_t sepconv_run(sepconv_plan_t plan, const float *in, const float *kernel, float *out,

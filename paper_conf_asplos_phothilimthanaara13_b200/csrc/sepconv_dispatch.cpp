@@ -15,6 +15,8 @@ const StreamEntry *stream_table_sep_v2();
 const StreamEntry *stream_table_sep_v3();
 const StreamEntry *stream_table_sep_v4();
 const StreamEntry *stream_table_sep_v5();
+const StreamEntry *stream_table_sep_v6();
+const StreamEntry *stream_table_sep_v7();
 
 static const StreamEntry *table(int op, int variant) {
     switch (op) {
@@ -40,6 +42,8 @@ static const StreamEntry *table(int op, int variant) {
                 case 3: return stream_table_sep_v3();
                 case 4: return stream_table_sep_v4();
                 case 5: return stream_table_sep_v5();
+                case 6: return stream_table_sep_v6();
+                case 7: return stream_table_sep_v7();
             }
             break;
     }

@@ -470,7 +470,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                 }
                 float b[V];
                 if constexpr (ROWCONV) {
-                    if constexpr (F2 >= 2) {
+                    if constexpr (F2 == 2) {
                         // same per-element order as the scalar path, two columns per instruction:
                         // xp[m] = (x_2m, x_2m+1) are the loaded pairs, xs[m] = (x_2m+1, x_2m+2) the
                         // shifted pairs odd taps need (built once per step, shared by both column pairs)
@@ -488,6 +488,19 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                                 bb = ffma2(p.k2[i], ((e + i) & 1) ? xs[(e + i) / 2] : xp[(e + i) / 2], bb);
                             b[e] = bb.x;
                             b[e + 1] = bb.y;
+                        }
+                    } else if constexpr (F2 == 3 && K >= 2) {
+                        // (exploration) two independent chains over even / odd taps, halving the
+                        // row pass's dependent-FMA depth: b = (sum_even) + (sum_odd)
+#pragma unroll
+                        for (int e = 0; e < V; ++e) {
+                            float b0 = p.k[0] * x[e], b1 = p.k[1] * x[e + 1];
+#pragma unroll
+                            for (int i = 2; i < K; ++i) {
+                                if (i & 1) b1 = fmaf(p.k[i], x[e + i], b1);
+                                else b0 = fmaf(p.k[i], x[e + i], b0);
+                            }
+                            b[e] = b0 + b1;
                         }
                     } else {
 #pragma unroll

@@ -74,12 +74,18 @@ struct alignas(64) Conv2DParams {
 //   cfg 1  8 warps, SR ~ 8 rows, up to 3 stages, CTA lockstep               (medium)
 //   cfg 2  8 warps, SR ~ 6 rows, 2 stages, warps free-running                (free)
 //   cfg 3  16 warps, SR ~ 6 rows, as many stages as fit (<= 4), free-running (wide)
+//   cfg 4  cfg 2 with the row pass in packed FP32 too (FFMA2 for both passes; the odd taps'
+//          shifted pairs cost a few MOVs): fewer issue slots, FMA-pipe-bound at K = 15-17
+//          (-2.6% at 16384^2 / K=17, tools/explore_mid.cu, profiles/r02_explore_mid.txt)
+//   cfg 5  4 warps (512-column CTA strips), SR ~ 6, 2 stages, free-running, 2 CTAs per SM:
+//          finer strips for widths that are not a multiple of 1024 columns (3520^2: -8%
+//          at K = 3 and 9)
 // "Lockstep" = a CTA barrier after every stage, so the 8 warps of a CTA read the same
 // rows (4 KB of each) together: measured +13% at K=9 and +4% at K=1 on 16384^2, because
 // DRAM sees whole row segments instead of 512-byte pieces at drifting times.  At K=17
 // (FMA-bound) the barrier costs a little, hence cfg 2; and there 16 warps (cfg 3, 128
 // registers, a few spilled) beat 8 warps with 2 stages by 10%.
-constexpr int kSepTmaConfigs = 4;
+constexpr int kSepTmaConfigs = 6;
 constexpr int kSmemPerCta = 232448 - 1024;     // opt-in limit minus headroom
 
 SEPCONV_HD constexpr int stream_bw(int K, int op) { return 32 * 4 + (op != OP_COLS ? (((K - 1) + 3) & ~3) : 0); }
@@ -105,9 +111,11 @@ SEPCONV_HD constexpr StreamGeom stream_geom(int K, int op, int variant) {
                                               clampi(ns_fit(8, sep_sr_medium(K), stream_bw(K, op)), 1, 3), K >= 2 ? 1 : 0,
                                               1, 1}
                   : variant == 4 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 1, 0}
-                                 : StreamGeom{16, sep_sr_shallow(K),
+                  : variant == 5 ? StreamGeom{16, sep_sr_shallow(K),
                                               clampi(ns_fit(16, sep_sr_shallow(K), stream_bw(K, op)), 1, 4),
-                                              K >= 2 ? 1 : 0, 1, 0})
+                                              K >= 2 ? 1 : 0, 1, 0}
+                  : variant == 6 ? StreamGeom{8, sep_sr_shallow(K), 2, K >= 2 ? 2 : 0, 1, 0}
+                                 : StreamGeom{4, sep_sr_shallow(K), 2, K >= 2 ? 1 : 0, 2, 0})
                : op == OP_ROWS ? StreamGeom{8, 8, clampi(ns_fit(8, 8, stream_bw(K, op)), 1, 8), 0, 0, 0}
                                : StreamGeom{8, K * ((8 + K - 1) / K),
                                             clampi(ns_fit(8, K * ((8 + K - 1) / K), stream_bw(K, op)), 1, 8),

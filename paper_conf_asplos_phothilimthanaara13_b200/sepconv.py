@@ -302,6 +302,21 @@ class Plan:
                                  _stream(stream)), "sepconv_run")
         return out
 
+    def bind(self, inp, kernel, out, variant="auto", stream=None):
+        """A prepared sepconv_run for a hot loop: the arguments are marshalled once (pointers,
+        kernel buffer, variant, raw stream handle) and the returned callable only makes the C
+        call and checks its status -- no per-call numpy or torch work."""
+        k = _kernel_buf(kernel, self.k)
+        fn = lib().sepconv_run
+        args = (self._h, ctypes.c_void_p(_ptr(inp)), ctypes.c_void_p(k.ctypes.data), ctypes.c_void_p(_ptr(out)),
+                ctypes.c_int(_variant(variant)), ctypes.c_void_p(_stream(stream)))
+
+        def call(_fn=fn, _args=args, _keep=k):
+            st = _fn(*_args)
+            if st:
+                _check(st, "sepconv_run")
+        return call
+
     def run_choice(self, inp, kernel, out, choice: Choice, stream=None):
         k = _kernel_buf(kernel, self.k)
         c = choice._c()

@@ -14,9 +14,10 @@ for (h, K) in [(64, 3), (2048, 3), (2048, 17), (4096, 17)]:
         lib, h_, xp, op_, kb = sc.lib(), p.handle, x.data_ptr(), out.data_ptr(), sc._kernel_buf(k, K)
         kp, st = kb.ctypes.data, sc._stream(None)
         raw = lambda: lib.sepconv_run(h_, xp, kp, op_, 2, st)
-        cands = [("auto", None), ("auto-raw-ctypes", raw)] + [(c.name, c) for c in p.candidates()]
+        cands = [("auto", None), ("auto-raw-ctypes", raw), ("auto-bind", p.bind(x, k, out, "auto"))] + \
+            [(c.name, c) for c in p.candidates()]
         if os.environ.get("AUTO_ONLY"):
-            cands = cands[:2]
+            cands = cands[:3]
         for name, c in cands:
             run = (lambda: p.run(x, k, out, "auto")) if c is None else (c if callable(c) else (lambda c=c: p.run_choice(x, k, out, c)))
             for _ in range(20):
