@@ -445,6 +445,9 @@ def main():
     def evpair():
         return torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
 
+    if flush:
+        for s in range(3):                        # first-call costs of the flush ops stay out of the timing
+            do_flush(s)
     ev = {K: [evpair() for _ in range(args.steps)] for K in widths}
     fev = {K: (evpair(), evpair()) for K in widths}
     e_start, e_end = evpair()
