@@ -58,6 +58,8 @@ def parse_args():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle time for the cpu_baseline sample")
     ap.add_argument("--tune-reps", type=int, default=10)
+    ap.add_argument("--tune-mutations", type=int, default=0,
+                    help="schedule mutations after the exhaustive tuning pass (0 = library default 12, -1 = none)")
     ap.add_argument("--sor-iters", type=int, default=24, help="poisson workload: iterations per step")
     ap.add_argument("--options", type=int, default=1 << 28, help="blackscholes workload: options per GPU")
     ap.add_argument("--dry-run", action="store_true",
@@ -404,7 +406,7 @@ def main():
     # ---- tune (the paper's install-time autotuning): per width, per rank ----
     choices = {}
     for K in widths:
-        choices[K] = plans[K].tune(reps=args.tune_reps)
+        choices[K] = plans[K].tune(reps=args.tune_reps, mutations=args.tune_mutations)
     torch.cuda.synchronize()
 
     def one_pass(K):

@@ -264,10 +264,16 @@ static Sched schedule_uncached(long long slots, int nimg, int nstrips, int rows,
 
 // The search above walks up to 2 x 4096 part counts (~10 us of host time at 16384^2): memoised
 // per (slots, images, strips, rows, K, mode), so a steady-state sepconv_run only looks it up.
-static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K) {
+static int sched_mode() {
     const char *mode = std::getenv("SEPCONV_SCHED");          // read per launch: tests flip it
-    const bool no_win = mode && std::strcmp(mode, "nowin") == 0;
-    const bool force_win = mode && std::strcmp(mode, "win") == 0;
+    if (!mode) return 0;
+    return std::strcmp(mode, "nowin") == 0 ? 1 : (std::strcmp(mode, "win") == 0 ? 2 : 0);
+}
+
+static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int rows, int K) {
+    const int mode = sched_mode();
+    const bool no_win = mode == 1;
+    const bool force_win = mode == 2;
     const long long slots = static_cast<long long>(di.sms) * occ;
     static std::mutex mu;
     static std::map<std::array<long long, 6>, Sched> memo;
@@ -303,7 +309,8 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
                                          long long ld_out, long long out_img, int out_cols, int rows_total,
                                          const float *kernel, bool want_tma, int cfg, int store_path,
                                          cudaStream_t st, int ov_parts = 0, int ov_grid = 0,
-                                         Sched *query = nullptr, long long *query_slots = nullptr) {
+                                         Sched *query = nullptr, long long *query_slots = nullptr,
+                                         sepconv_plan_s::Replay *record = nullptr) {
     const int K = g.K;
     const bool tma = want_tma && tma_ok(in, ld_in, in_img);
     const bool vec = aligned(in, 16) && (ld_in % 4) == 0 && (in_img % 4) == 0;
@@ -360,6 +367,14 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     cudaError_t e = stream_launch(op, map, K, smode, p, sc.grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
+    if (record) {
+        record->op = op;
+        record->map = map;
+        record->smode = smode;
+        record->grid = sc.grid;
+        record->p = p;
+        record->valid = true;
+    }
     return SEPCONV_OK;
 }
 
@@ -637,6 +652,8 @@ void sepconv_destroy(sepconv_plan_t plan) {
         for (auto &ev : row)
             if (ev) cudaEventDestroy(ev);
     if (plan->last_work) cudaEventDestroy(plan->last_work);
+    for (auto &e : plan->tev)
+        if (e) cudaEventDestroy(e);
     delete plan;
 }
 
@@ -685,9 +702,44 @@ static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const
         if (s != SEPCONV_OK) return s;
     }
     Geometry g = plan_geometry(plan);
-    // the unfused buffer for a whole-image launch is [n][h][ld_buf] (rows = ho + K - 1 = h)
     // (no per-call event: sepconv_destroy synchronises the device before freeing anything)
-    return launch_candidate(plan, g, in, out, kernel, c, plan->buf, plan->ld_buf, st);
+    if (!(c.algo == SEPCONV_SEPARABLE && c.fused))
+        // the unfused buffer for a whole-image launch is [n][h][ld_buf] (rows = ho + K - 1 = h)
+        return launch_candidate(plan, g, in, out, kernel, c, plan->buf, plan->ld_buf, st);
+    // fused separable: replay the last launch's parameter block when nothing but the weights can
+    // have changed (same pointers, candidate and schedule mode); else build it and record it
+    sepconv_plan_s::Replay &r = plan->replay;
+    const int mode = sched_mode();
+    if (r.valid && r.in == in && r.out == out && r.algo == c.algo && r.mapping == c.mapping && r.fused == c.fused &&
+        r.config == c.config && r.store == c.store && r.sched_parts == c.sched_parts &&
+        r.sched_grid == c.sched_grid && r.sched_mode == mode) {
+        for (int i = 0; i < plan->k; ++i) {
+            r.p.k[i] = kernel[i];
+            r.p.k2[i] = make_float2(kernel[i], kernel[i]);
+        }
+        if (r.p.total <= 0) return SEPCONV_OK;
+        cudaError_t e = stream_launch(r.op, r.map, plan->k, r.smode, r.p, r.grid, st);
+        if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
+        g_launches.fetch_add(1, std::memory_order_relaxed);
+        return SEPCONV_OK;
+    }
+    r.valid = false;
+    s = launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img, g.out_cols,
+                         g.rows, kernel, c.mapping == SEPCONV_MAP_TMA, c.config, c.store, st, c.sched_parts,
+                         c.sched_grid, nullptr, nullptr, &r);
+    if (s == SEPCONV_OK && r.valid) {
+        r.in = in;
+        r.out = out;
+        r.algo = c.algo;
+        r.mapping = c.mapping;
+        r.fused = c.fused;
+        r.config = c.config;
+        r.store = c.store;
+        r.sched_parts = c.sched_parts;
+        r.sched_grid = c.sched_grid;
+        r.sched_mode = mode;
+    }
+    return s;
 }
 
 sepconv_status_t sepconv_run(sepconv_plan_t plan, const float *in, const float *kernel, float *out,

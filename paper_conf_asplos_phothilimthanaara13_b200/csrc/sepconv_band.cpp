@@ -18,6 +18,8 @@
 #include <mutex>
 #include <string>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "sepconv_internal.h"
 
 using namespace sepconv;
@@ -141,6 +143,17 @@ void sepconv_comm_destroy_internal(sepconv_plan_t plan) {
     plan->band_external = false;
 }
 
+// NVTX range on the host timeline (visible to nsys / ncu --nvtx); popped once
+struct NvtxScope {
+    bool open = true;
+    explicit NvtxScope(const char *name) { nvtxRangePushA(name); }
+    void end() {
+        if (open) nvtxRangePop();
+        open = false;
+    }
+    ~NvtxScope() { end(); }
+};
+
 extern "C" {
 
 sepconv_status_t sepconv_band(int64_t H, int K, int G, int g, int64_t *out_row0, int64_t *out_rows,
@@ -225,9 +238,16 @@ sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const flo
         if (s != SEPCONV_OK) return s;
     }
 
+    // timeline events (sepconv_band_trace): [0] start, [1,2] interior, [3,4] exchange, [5,6] tail
+    cudaEvent_t *tv = plan->trace ? plan->tev : nullptr;
+    NvtxScope whole("sepconv_run_band");
+    if (tv) SC_CUDA(cudaEventRecord(tv[0], st));
+
     // 1. the exchange (comm stream, after the caller's writes to in_band on `st`)
     SC_CUDA(cudaEventRecord(plan->ev_in, st));
     SC_CUDA(cudaStreamWaitEvent(plan->comm_stream, plan->ev_in, 0));
+    if (tv) SC_CUDA(cudaEventRecord(tv[3], plan->comm_stream));
+    NvtxScope xchg("halo exchange (NCCL send/recv)");
     if (halo > 0 && plan->nranks > 1 && !plan->band_external) {
         const size_t cnt = static_cast<size_t>(halo) * plan->ld_in;
         nccl_comm_t comm = static_cast<nccl_comm_t>(plan->comm);
@@ -240,11 +260,15 @@ sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const flo
         if (r != 0) return nccl_fail(r, "ncclSend/ncclRecv");
         if (r2 != 0) return nccl_fail(r2, "ncclGroupEnd");
     }
+    if (tv) SC_CUDA(cudaEventRecord(tv[4], plan->comm_stream));
     SC_CUDA(cudaEventRecord(plan->ev_halo, plan->comm_stream));
+    xchg.end();
 
     // 2. interior rows: need only owned input rows, overlap the exchange
     Geometry g = plan_geometry(plan);
     const int64_t interior = last ? ho : ho - halo;
+    NvtxScope inner("interior rows");
+    if (tv) SC_CUDA(cudaEventRecord(tv[1], st));
     if (interior > 0) {
         Geometry gi = g;
         gi.row_begin = 0;
@@ -252,9 +276,13 @@ sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const flo
         s = launch_candidate(plan, gi, in_band, out_band, kernel, c, plan->buf, plan->ld_buf, st);
         if (s != SEPCONV_OK) return s;
     }
+    if (tv) SC_CUDA(cudaEventRecord(tv[2], st));
+    inner.end();
     // 3. tail rows after the halo has landed (and, on every rank, after our send
     //    has read in_band, so the caller may reuse it in stream order)
+    NvtxScope tail("tail rows (after the halo)");
     SC_CUDA(cudaStreamWaitEvent(st, plan->ev_halo, 0));
+    if (tv) SC_CUDA(cudaEventRecord(tv[5], st));
     if (!last && halo > 0) {
         Geometry gt = g;
         gt.row_begin = static_cast<int>(interior);
@@ -262,8 +290,29 @@ sepconv_status_t sepconv_run_band(sepconv_plan_t plan, float *in_band, const flo
         s = launch_candidate(plan, gt, in_band, out_band, kernel, c, plan->buf, plan->ld_buf, st);
         if (s != SEPCONV_OK) return s;
     }
+    if (tv) SC_CUDA(cudaEventRecord(tv[6], st));
     SC_CUDA(cudaEventRecord(plan->last_work, st));
     if (prev >= 0 && prev != plan->dev.device) cudaSetDevice(prev);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_band_trace(sepconv_plan_t plan, int enable) {
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
+    int prev = -1;
+    cudaGetDevice(&prev);
+    SC_CUDA(cudaSetDevice(plan->dev.device));
+    if (enable && !plan->tev[0])
+        for (auto &e : plan->tev) SC_CUDA(cudaEventCreate(&e));
+    plan->trace = enable != 0;
+    if (prev >= 0) cudaSetDevice(prev);
+    return SEPCONV_OK;
+}
+
+sepconv_status_t sepconv_band_timeline(sepconv_plan_t plan, float ms[6]) {
+    if (!plan || !ms) return fail(SEPCONV_E_INVALID, "NULL argument");
+    if (!plan->trace || !plan->tev[0]) return fail(SEPCONV_E_INVALID, "sepconv_band_trace is not enabled on this plan");
+    SC_CUDA(cudaEventSynchronize(plan->tev[6]));
+    for (int i = 0; i < 6; ++i) SC_CUDA(cudaEventElapsedTime(&ms[i], plan->tev[0], plan->tev[i + 1]));
     return SEPCONV_OK;
 }
 

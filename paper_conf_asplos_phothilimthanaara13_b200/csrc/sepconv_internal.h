@@ -96,6 +96,19 @@ struct sepconv_plan_s {
     sepconv_choice_t best[3] = {};
 
     sepconv::TensorMapCache tmaps;
+
+    // replay record of the last whole-plan single-kernel streaming launch (sepconv_run's fast
+    // path): the same pointers, candidate and schedule mode reuse its parameter block, grid and
+    // kernel, refreshing only the weights
+    struct Replay {
+        bool valid = false;
+        const float *in = nullptr;
+        float *out = nullptr;
+        int algo = -1, mapping = -1, fused = -1, config = -1, store = -1, sched_parts = 0, sched_grid = 0;
+        int sched_mode = 0;                 // $SEPCONV_SCHED at record time
+        int op = 0, map = 0, smode = 0, grid = 0;
+        sepconv::StreamParams p;
+    } replay;
     cudaEvent_t last_work = nullptr;
 
     // NCCL (row bands)
@@ -104,6 +117,10 @@ struct sepconv_plan_s {
     int nranks = 1, rank = 0;
     cudaStream_t comm_stream = nullptr;
     cudaEvent_t ev_in = nullptr, ev_halo = nullptr;
+    // band timeline (sepconv_band_trace): timing events t0, interior start/end, exchange
+    // start/end (comm stream), tail start/end of the last sepconv_run_band
+    bool trace = false;
+    cudaEvent_t tev[7] = {};
 
     // host-resident pipeline
     cudaStream_t hstream[3] = {nullptr, nullptr, nullptr};

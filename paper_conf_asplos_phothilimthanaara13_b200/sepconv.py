@@ -168,6 +168,8 @@ def lib() -> ctypes.CDLL:
             "sepconv_nccl_unique_id": (I, [ctypes.c_char_p]),
             "sepconv_comm_init": (I, [P, ctypes.c_char_p, I, I]),
             "sepconv_run_band": (I, [P, P, P, P, I, P]),
+            "sepconv_band_trace": (I, [P, I]),
+            "sepconv_band_timeline": (I, [P, ctypes.POINTER(ctypes.c_float)]),
             "sepconv_status_str": (ctypes.c_char_p, [I]),
             "sepconv_last_error": (ctypes.c_char_p, []),
             "sepconv_version": (ctypes.c_char_p, []),
@@ -201,7 +203,8 @@ def exported_symbols():
             "sepconv_run_choice", "sepconv_run_host", "sepconv_tune", "sepconv_tune_selector", "sepconv_select",
             "sepconv_get_choice",
             "sepconv_num_candidates", "sepconv_get_candidate", "sepconv_band", "sepconv_nccl_unique_id",
-            "sepconv_comm_init", "sepconv_run_band", "sepconv_status_str", "sepconv_last_error",
+            "sepconv_comm_init", "sepconv_run_band", "sepconv_band_trace", "sepconv_band_timeline",
+            "sepconv_status_str", "sepconv_last_error",
             "sepconv_version", "sepconv_launch_count"]
 
 
@@ -360,6 +363,16 @@ class Plan:
         if unique_id is not None and len(unique_id) != NCCL_ID_BYTES:
             raise ValueError("NCCL unique id must be 128 bytes")
         _check(lib().sepconv_comm_init(self._h, unique_id, int(nranks), int(rank)), "sepconv_comm_init")
+
+    def band_trace(self, enable: bool = True):
+        """sepconv_band_trace: record the phase timeline of later run_band calls."""
+        _check(lib().sepconv_band_trace(self._h, int(bool(enable))), "sepconv_band_trace")
+
+    def band_timeline(self):
+        """sepconv_band_timeline: {interior, exchange, tail: (start_ms, end_ms)} of the last run_band."""
+        ms = (ctypes.c_float * 6)()
+        _check(lib().sepconv_band_timeline(self._h, ms), "sepconv_band_timeline")
+        return {"interior": (ms[0], ms[1]), "exchange": (ms[2], ms[3]), "tail": (ms[4], ms[5])}
 
     def run_band(self, in_band, kernel, out_band, variant="auto", stream=None):
         k = _kernel_buf(kernel, self.k)

@@ -317,6 +317,61 @@ def test_run_band_external_halo_equals_whole_image(G, K):
         assert torch.equal(got, want), v
 
 
+def test_repeated_calls_refresh_weights_and_choices():
+    """sepconv_run's replay fast path (same plan and pointers) must still take each call's
+    weights, candidate and schedule: alternate kernels, fused configurations and schedule
+    overrides on the same buffers, every result checked against the oracle or bitwise."""
+    h, w, K = 700, 1500, 9
+    img = synth.uniform_image(h, w, seed=17)
+    dev = torch.from_numpy(img).cuda()
+    out = torch.empty((h - K + 1, w - K + 1), device="cuda")
+    p = sc.Plan(h, w, K)
+    ka, kb = synth.random_kernel(K, seed=1, signed=True), synth.random_kernel(K, seed=2, signed=True)
+    for k in (ka, kb, ka):
+        out.fill_(float("nan"))
+        p.run(dev, k, out, "separable")
+        torch.cuda.synchronize()
+        check(img, k, out.cpu().numpy())
+    ref = out.clone()
+    for cfg in range(6):
+        for parts in (0, 3):
+            out.fill_(float("nan"))
+            p.run_choice(dev, ka, out, sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, sched_parts=parts))
+            torch.cuda.synchronize()
+            assert torch.equal(out, ref), (cfg, parts)
+    run = p.bind(dev, kb, out, "separable")
+    for _ in range(3):
+        run()
+    torch.cuda.synchronize()
+    check(img, kb, out.cpu().numpy())
+
+
+def test_band_timeline_orders_the_phases():
+    """sepconv_band_trace / sepconv_band_timeline (the overlap evidence of SURVEY 8(e)): on a
+    middle band in external-halo mode the interior kernel, the (empty) exchange and the tail
+    kernel are timed on the device; the tail starts after the interior ends and after the
+    exchange event, every interval is non-negative, and tracing changes no output bit."""
+    H, W, K, G, g = 3000, 4096, 9, 3, 1
+    img = torch.from_numpy(synth.uniform_image(H, W, seed=43)).cuda()
+    k = synth.binomial_kernel(K)
+    r0, rows, owned, alloc = sc.band(H, K, G, g)
+    band = img[r0:r0 + alloc].clone()
+    p = sc.Plan(alloc, W, K)
+    p.comm_init(None, G, g)
+    with pytest.raises(sc.SepconvError):
+        p.band_timeline()                                 # tracing off
+    out0 = torch.empty((rows, W - K + 1), device="cuda")
+    p.run_band(band, k, out0)
+    p.band_trace(True)
+    out1 = torch.empty_like(out0)
+    p.run_band(band, k, out1)
+    tl = p.band_timeline()
+    (i0, i1), (x0, x1), (t0, t1) = tl["interior"], tl["exchange"], tl["tail"]
+    assert 0 <= i0 <= i1 and 0 <= x0 <= x1 and 0 <= t0 <= t1
+    assert t0 >= i1 and t0 >= x1 and i1 - i0 > 0 and t1 - t0 > 0
+    assert torch.equal(out0, out1)
+
+
 def test_run_band_nccl_single_rank_and_shared_comm():
     """The NCCL path end to end on one GPU: the library dlopens the process's libnccl,
     creates a unique id and a 1-rank communicator (no peers, so no send/recv is posted),
