@@ -176,6 +176,48 @@ class ClockSampler:
 
 
 # --------------------------------------------------------------------------------------------
+class CleanFlush:
+    """The L2 flush between timed passes when the working set fits in L2: write a 2 x L2 scratch
+    buffer, then read a second 2 x L2 buffer, so the pass starts from an L2 of clean, unrelated
+    lines (a write alone leaves ~L2-size of dirty lines whose write-back the next pass would pay,
+    profiles/r02_flush_study.txt)."""
+
+    def __init__(self, torch, dev):
+        l2 = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
+        self.torch = torch
+        self.w = torch.empty(2 * l2 // 4, dtype=torch.float32, device=dev)
+        self.r = torch.zeros(2 * l2 // 4, dtype=torch.float32, device=dev)
+        self.sink = torch.empty((), dtype=torch.float32, device=dev)
+        for i in range(3):                       # first-call costs stay out of any timing
+            self(i)
+
+    def __call__(self, i=0):
+        self.w.fill_(float(i))
+        self.torch.sum(self.r, dim=0, out=self.sink)
+
+    LABEL = ("L2 flushed before every step (write 2 x L2, then read another 2 x L2 so L2 holds clean unrelated "
+             "lines); step time = [events around steps x (flush + step)] - [events around steps x flush], / steps")
+
+
+def time_flushed(torch, stream, steps, body, flush):
+    """Marginal device ms of `body` after a clean flush, from two event-timed batches: single event
+    pairs around a short pass read a ~5 us event/launch floor in 2.048 us ticks
+    (profiles/r02_latency_probe.txt)."""
+    a0, a1, b0, b1 = (torch.cuda.Event(enable_timing=True) for _ in range(4))
+    a0.record(stream)
+    for i in range(steps):
+        flush(i)
+        body()
+    a1.record(stream)
+    b0.record(stream)
+    for i in range(steps):
+        flush(i)
+    b1.record(stream)
+    torch.cuda.synchronize()
+    return max(1e-6, a0.elapsed_time(a1) - b0.elapsed_time(b1)) / steps
+
+
+# --------------------------------------------------------------------------------------------
 def oracle_sample(img_rows_fn, W, widths, target_s, nthreads=0, H=None):
     """Time the oracle (as it stands) on the first S output rows of the image for every width;
     an image with fewer rows than the sample needs is convolved whole, `reps` times over."""
@@ -323,10 +365,10 @@ def main():
         return run_dry(args)
     if args.workload == "poisson":
         import bench_poisson
-        return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit)
+        return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed))
     if args.workload == "blackscholes":
         import bench_bs
-        return bench_bs.run(args, peaks, dist_env, ClockSampler, emit)
+        return bench_bs.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed))
     if args.impl == "reference":
         return run_reference(args)
 

@@ -38,7 +38,7 @@ def _oracle_sample(target_s: float):
             "sample": f"{reps} x {n} options (oracle_black_scholes, double, one thread), {el:.1f} s"}
 
 
-def run(args, peaks_fn, dist_env, ClockSampler, emit):
+def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
     world, rank, local = dist_env()
     if args.impl == "reference":
         if rank != 0:
@@ -84,25 +84,29 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
     if dist:
         dist.barrier()
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
-    # a working set that fits in L2 (the paper's 500000 options: 10 MB) is flushed before every
-    # step by a 2 x L2 torch fill outside the events
+    # a working set that fits in L2 (the paper's 500000 options: 10 MB) gets a clean flush before
+    # every step and is timed as a batched difference (bench.py CleanFlush / time_flushed)
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = 20 * n <= 2 * l2_bytes
-    scratch = torch.empty(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
+    CleanFlush, time_flushed = flushing
+    flusher = CleanFlush(torch, dev) if flush else None
     launches0 = sc.launch_count()
     with ClockSampler(local) as clk:
         torch.cuda.synchronize()
         torch.cuda.nvtx.range_push("sepconv_timed")
-        for i in range(args.steps):
-            if flush:
-                scratch.fill_(float(i))
-            ev[i][0].record(stream)
-            bs.price(ds, dx, dt, r, v, dc, dp, stream=stream)
-            ev[i][1].record(stream)
+        if flush:
+            ms = time_flushed(torch, stream, args.steps,
+                              lambda: bs.price(ds, dx, dt, r, v, dc, dp, stream=stream), flusher)
+        else:
+            for i in range(args.steps):
+                ev[i][0].record(stream)
+                bs.price(ds, dx, dt, r, v, dc, dp, stream=stream)
+                ev[i][1].record(stream)
         torch.cuda.nvtx.range_pop()
         torch.cuda.synchronize()
     launches = sc.launch_count() - launches0
-    ms = statistics.median(a.elapsed_time(b) for a, b in ev)
+    if not flush:
+        ms = statistics.median(a.elapsed_time(b) for a, b in ev)
     if dist:
         tt = torch.tensor([ms], dtype=torch.float64, device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
@@ -144,8 +148,7 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
               "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
               "vs_baseline": None, "dtype": "f32", "data": "synthetic",
               "config": {"workload": f"Black-Scholes, {n} float32 options per GPU (r={r}, v={v})",
-                         "options": n, "l2": ("L2 flushed before every step (2 x L2 write outside the events)" if flush
-                                               else "inputs larger than L2 (no flush)"),
+                         "options": n, "l2": CleanFlush.LABEL if flush else "inputs larger than L2 (no flush)",
                          "parallelism": f"options sharded x{world}" if world > 1 else "1 GPU"},
               "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
               "clocks": clk.summary()})

@@ -39,7 +39,7 @@ def _oracle_sample(target_s: float):
             "sample": f"{n}x{n} grid, {iters} red-black iterations in double (oracle_sor_rb, one thread), {t:.1f} s"}
 
 
-def run(args, peaks_fn, dist_env, ClockSampler, emit):
+def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
     if args.impl == "reference":
         world, rank, _ = dist_env()
         if rank != 0:
@@ -119,25 +119,29 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
     if dist:
         dist.barrier()
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
-    # a working set that fits in L2 (six split buffers) is flushed between steps by a 2 x L2
-    # torch fill outside the events; inside a step the iterations reuse L2 as the method does
+    # a working set that fits in L2 (six split buffers) gets a clean flush between steps and is
+    # timed as a batched difference (bench.py CleanFlush / time_flushed); inside a step the
+    # iterations reuse L2 as the method does
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = 6 * rows * n * 4 <= 2 * l2_bytes          # n columns (square grid)
-    scratch = torch.empty(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
+    CleanFlush, time_flushed = flushing
+    flusher = CleanFlush(torch, dev) if flush else None
     launches0 = sc.launch_count()
     with ClockSampler(local) as clk:
         torch.cuda.synchronize()
         torch.cuda.nvtx.range_push("sepconv_timed")
-        for i in range(args.steps):
-            if flush:
-                scratch.fill_(float(i))
-            ev[i][0].record(stream)
-            step()
-            ev[i][1].record(stream)
+        if flush:
+            ms = time_flushed(torch, stream, args.steps, step, flusher)
+        else:
+            for i in range(args.steps):
+                ev[i][0].record(stream)
+                step()
+                ev[i][1].record(stream)
         torch.cuda.nvtx.range_pop()
         torch.cuda.synchronize()
     launches = sc.launch_count() - launches0
-    ms = statistics.median(a.elapsed_time(c) for a, c in ev)
+    if not flush:
+        ms = statistics.median(a.elapsed_time(c) for a, c in ev)
     if dist:
         t = torch.tensor([ms], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
@@ -195,8 +199,8 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit):
               "config": {"workload": f"Poisson2D red-black SOR, {n}x{n} float32 grid, {iters} iterations per step",
                          "grid": [n, n], "iters_per_step": iters, "omega": omega,
                          "variant": "auto (tuned): " + ("half" if variant_id == sor.SOR_HALF else f"wave depth {depth}"),
-                         "l2": ("L2 flushed between steps (2 x L2 write outside the events; the iterations of a step "
-                                "reuse L2)") if flush else "grid larger than L2 (no flush)",
+                         "l2": (CleanFlush.LABEL + "; the iterations of a step reuse L2") if flush
+                         else "grid larger than L2 (no flush)",
                          "parallelism": (f"row bands x{world}, {2 * depth}-row ghost exchange per pass (NCCL)"
                                          if world > 1 else "1 GPU")},
               "gcell_it_s": value / 1e3, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
