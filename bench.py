@@ -196,25 +196,35 @@ class CleanFlush:
         self.torch.sum(self.r, dim=0, out=self.sink)
 
     LABEL = ("L2 flushed before every step (write 2 x L2, then read another 2 x L2 so L2 holds clean unrelated "
-             "lines); step time = [events around steps x (flush + step)] - [events around steps x flush], / steps")
+             "lines); step time = [events around steps x (flush + step)] - [mean of events around steps x flush "
+             "before and after], / steps, after a spin-up of 20 flushes")
 
 
 def time_flushed(torch, stream, steps, body, flush):
-    """Marginal device ms of `body` after a clean flush, from two event-timed batches: single event
-    pairs around a short pass read a ~5 us event/launch floor in 2.048 us ticks
-    (profiles/r02_latency_probe.txt)."""
-    a0, a1, b0, b1 = (torch.cuda.Event(enable_timing=True) for _ in range(4))
-    a0.record(stream)
+    """Marginal device ms of `body` after a clean flush: events around `steps` x [flush, body]
+    minus the mean of event-timed `steps` x [flush] batches run just before and just after it
+    (single event pairs around a short pass read a ~5 us event/launch floor in 2.048 us ticks,
+    profiles/r02_latency_probe.txt).  A spin-up of flushes first brings the clocks up from idle,
+    so the first batch is not timed on a ramping GPU."""
+    ev = [torch.cuda.Event(enable_timing=True) for _ in range(6)]
+    for i in range(20):
+        flush(i)
+    ev[0].record(stream)
+    for i in range(steps):
+        flush(i)
+    ev[1].record(stream)
+    ev[2].record(stream)
     for i in range(steps):
         flush(i)
         body()
-    a1.record(stream)
-    b0.record(stream)
+    ev[3].record(stream)
+    ev[4].record(stream)
     for i in range(steps):
         flush(i)
-    b1.record(stream)
+    ev[5].record(stream)
     torch.cuda.synchronize()
-    return max(1e-6, a0.elapsed_time(a1) - b0.elapsed_time(b1)) / steps
+    t_flush = 0.5 * (ev[0].elapsed_time(ev[1]) + ev[4].elapsed_time(ev[5]))
+    return max(1e-6, ev[2].elapsed_time(ev[3]) - t_flush) / steps
 
 
 # --------------------------------------------------------------------------------------------
@@ -474,26 +484,17 @@ def main():
     # +2-6 us, profiles/r02_flush_study.txt).  A single event pair around one short pass measures
     # a ~5 us event/launch floor in 2.048 us ticks (profiles/r02_latency_probe.txt), so per
     # width the flushed mode times `steps` x [flush, pass] and `steps` x [flush] between event
-    # pairs and takes the difference: the marginal device time of the pass inside a stream of
-    # work, as the unflushed mode measures it.
+    # pairs and takes the difference (time_flushed): the marginal device time of the pass inside
+    # a stream of work, as the unflushed mode measures it.
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
-    scratch = torch.empty(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
-    rscratch = torch.zeros(2 * l2_bytes // 4, dtype=torch.float32, device=dev) if flush else None
-    sink = torch.empty((), dtype=torch.float32, device=dev)
-
-    def do_flush(s):
-        scratch.fill_(float(s))
-        torch.sum(rscratch, dim=0, out=sink)
+    do_flush = CleanFlush(torch, dev) if flush else None
 
     def evpair():
         return torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
 
-    if flush:
-        for s in range(3):                        # first-call costs of the flush ops stay out of the timing
-            do_flush(s)
     ev = {K: [evpair() for _ in range(args.steps)] for K in widths}
-    fev = {K: (evpair(), evpair()) for K in widths}
+    per_k_ms = {}
     e_start, e_end = evpair()
     launches0 = sc.launch_count()
     with ClockSampler(local) as clk:
@@ -504,16 +505,7 @@ def main():
         e_start.record(stream)
         if flush:
             for K in widths:
-                (a0, a1), (b0, b1) = fev[K]
-                a0.record(stream)
-                for s in range(args.steps):
-                    do_flush(s)
-                    one_pass(K)
-                a1.record(stream)
-                b0.record(stream)
-                for s in range(args.steps):
-                    do_flush(s)
-                b1.record(stream)
+                per_k_ms[K] = time_flushed(torch, stream, args.steps, lambda K=K: one_pass(K), do_flush)
         else:
             for s in range(args.steps):
                 for K in widths:
@@ -531,8 +523,6 @@ def main():
         dist.all_reduce(tl)
         launches = int(tl.item())
     if flush:                                    # the flushes are not part of the step
-        per_k_ms = {K: max(1e-6, fev[K][0][0].elapsed_time(fev[K][0][1]) - fev[K][1][0].elapsed_time(fev[K][1][1]))
-                    / args.steps for K in widths}
         total_ms = sum(per_k_ms.values()) * args.steps
     else:
         total_ms = e_start.elapsed_time(e_end)
@@ -665,9 +655,7 @@ def main():
                             if args.workload == "image" else f"{N_img} x {H}x{W} float32 images, width 11"),
                "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
                "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
-               "l2": ("L2 flushed before every pass (write 2 x L2, then read another 2 x L2 so L2 holds clean "
-                      "unrelated lines); per width, pass time = [events around steps x (flush + pass)] - "
-                      "[events around steps x flush], / steps; ms_per_step = sum over widths")
+               "l2": (CleanFlush.LABEL.replace("step", "pass") + "; per width; ms_per_step = sum over widths")
                if flush else "inputs larger than L2 (no flush)",
                "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
                                else f"images sharded x{world}" if world > 1 else "1 GPU")}
