@@ -83,7 +83,8 @@ sepconv_status_t sor_solve_host(sor_plan_t plan, const float *x, const float *b,
 sepconv_status_t sor_buffers(sor_plan_t plan, float **u_red, float **u_black, float **b_red, float **b_black,
                              int64_t *ldh);
 
-/* Empirical choice between SOR_HALF and SOR_WAVE (wavefront depths 1..8) for this
+/* Empirical choice between SOR_HALF and SOR_WAVE (wavefront depths 1..8, each with 1, 1/2
+ * or 1/3 row segments per resident warp -- the wave schedule's size-like tunable) for this
  * grid at `iters_hint` iterations: median of `reps` event-timed runs on the legacy
  * default stream (synchronous).  It iterates the plan's own buffers, so call it
  * before sor_load (or load again afterwards).  Writes the chosen variant and depth

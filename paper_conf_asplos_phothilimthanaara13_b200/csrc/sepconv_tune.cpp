@@ -435,6 +435,29 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
     if ((status = b.open(plan, !(flags & SEPCONV_TUNE_NO_L2_FLUSH))) != SEPCONV_OK) return status;
     for (size_t ci = 0; ci < cs.size(); ++ci)
         if ((status = b.time(cs[ci], reps, &med[ci])) != SEPCONV_OK) return status;
+    // finalists -- up to four candidates within 8% of the fastest -- are timed twice more in
+    // interleaved rounds and keep the median of their three measurements: one sequential pass
+    // over the candidates picked a configuration 8% slower than the runner-up on 16384^2 / K=13
+    // (a transient during the runner-up's batches; profiles/r02_interleave.txt)
+    {
+        const float fastest = *std::min_element(med.begin(), med.end());
+        std::vector<size_t> fin;
+        for (size_t i = 0; i < cs.size(); ++i)
+            if (med[i] >= 0 && med[i] <= fastest * 1.08f) fin.push_back(i);
+        std::sort(fin.begin(), fin.end(), [&](size_t a, size_t c) { return med[a] < med[c]; });
+        if (fin.size() > 4) fin.resize(4);
+        if (fin.size() > 1) {
+            std::vector<float> t1(fin.size()), t2(fin.size());
+            for (int round = 0; round < 2; ++round)
+                for (size_t f = 0; f < fin.size(); ++f)
+                    if ((status = b.time(cs[fin[f]], reps, round ? &t2[f] : &t1[f])) != SEPCONV_OK) return status;
+            for (size_t f = 0; f < fin.size(); ++f) {
+                float v[3] = {med[fin[f]], t1[f], t2[f]};
+                std::sort(v, v + 3);
+                med[fin[f]] = v[1];
+            }
+        }
+    }
 
     auto better = [&](size_t a, size_t c) {   // is candidate a better than incumbent c?
         if (med[a] < 0) return false;

@@ -445,6 +445,7 @@ struct sor_plan_s {
     float *b[2] = {};
     int cur = 0;                     // pair holding the current iterate
     int variant = -1, depth = 0;     // tuned (variant < 0: untuned)
+    int seg_div = 1;                 // wave schedule: row segments = (resident warps / strips) / seg_div (tuned)
     int forced_depth = 0;
     int wave_occ[sor::kMaxDepth + 1] = {};
     CUtensorMap tmap;                // {ldh, n, 6} over buf (the wave kernel's TMA source)
@@ -531,15 +532,17 @@ sepconv_status_t wave_pass(sor_plan_t plan, float omega, int T, cudaStream_t st)
         if (e != cudaSuccess) return cuda_fail(e, "sor wave occupancy");
         occ = std::max(occ, 1);
     }
-    // items = strips x row segments, about one per resident warp.  Each segment pays ~4T
-    // warm-up/drain steps, but idle warps cost more: on the paper's 2048^2 a floor of 16T rows
-    // per segment left three quarters of the warps idle (372 G vs 565 G cell-it/s at T=3,
-    // profiles/r01_sor_perf.txt), so segments only keep >= 2T rows.  Segment rows are a multiple
+    // items = strips x row segments, about one per resident warp (/ seg_div, which sor_tune
+    // sets: fewer, longer segments trade idle warps for less warm-up, and fewer warps per SM
+    // each issue faster).  Each segment pays ~4T warm-up/drain steps, but idle warps cost more:
+    // on the paper's 2048^2 a floor of 16T rows per segment left three quarters of the warps
+    // idle (372 G vs 565 G cell-it/s at T=3, profiles/r01_sor_perf.txt), so segments only keep
+    // >= 2T rows.  Segment rows are a multiple
     // of the 6-step unroll, so every segment starts on a block boundary and no steps are wasted
     // aligning its first block.
     p.nstrips = static_cast<int>((plan->ldh + sor::kWout[T] - 1) / sor::kWout[T]);
     const long long warps = static_cast<long long>(plan->sms) * occ * sor::kWaveWarps;
-    long long nsegs = std::max<long long>(1, warps / p.nstrips);
+    long long nsegs = std::max<long long>(1, warps / p.nstrips / std::max(1, plan->seg_div));
     nsegs = std::min<long long>(nsegs, std::max<long long>(1, plan->n / (2 * T)));
     p.seg_rows = static_cast<int>(((plan->n + nsegs - 1) / nsegs + 5) / 6 * 6);
     nsegs = (plan->n + p.seg_rows - 1) / p.seg_rows;
@@ -858,11 +861,15 @@ sepconv_status_t sor_tune(sor_plan_t plan, int iters_hint, int reps, int *varian
     SC_CUDA(cudaEventCreate(&e0));
     SC_CUDA(cudaEventCreate(&e1));
     const int depths[] = {0, 1, 2, 3, 4, 5, 6, 8};       // 0 = SOR_HALF
+    const int divs[] = {1, 2, 3};                         // wave segments per resident warp: 1, 1/2, 1/3
     float best = 1e30f;
-    int best_v = SOR_WAVE, best_d = kDefaultDepth;
+    int best_v = SOR_WAVE, best_d = kDefaultDepth, best_div = 1;
     const float omega = 1.5f;
     sepconv_status_t status = SEPCONV_OK;
-    for (int d : depths) {
+    for (int cand = 0; cand < 8 * 3 && status == SEPCONV_OK; ++cand) {
+        const int d = depths[cand / 3], div = divs[cand % 3];
+        if (d == 0 && div != 1) continue;
+        plan->seg_div = div;
         float times[64];
         const int R = std::min(reps, 64);
         for (int r = -1; r < R && status == SEPCONV_OK; ++r) {
@@ -882,10 +889,12 @@ sepconv_status_t sor_tune(sor_plan_t plan, int iters_hint, int reps, int *varian
             best = med;
             best_v = d == 0 ? SOR_HALF : SOR_WAVE;
             best_d = d == 0 ? kDefaultDepth : d;
+            best_div = div;
         }
     }
     cudaEventDestroy(e0);
     cudaEventDestroy(e1);
+    plan->seg_div = best_div;
     if (status != SEPCONV_OK) return status;
     plan->variant = best_v;
     plan->depth = best_d;
