@@ -547,7 +547,7 @@ def main():
     for K in widths:
         t_s = per_k_ms[K] * 1e-3
         gbs = alg_bytes(K) / t_s / 1e9
-        per_width[str(K)] = {"variant": choices[K].name,
+        per_width[str(K)] = {"variant": choices[K].name, "tuned_us": choices[K].median_us,
                              "us": per_k_ms[K] * 1e3, "mpix_s": out_px_job[K] / t_s / 1e6, "gbs": gbs,
                              "frac_of_measured": gbs / (peak_gbs * world),
                              "frac_of_8tbs": gbs / (NOMINAL_HBM_GBS * world)}

@@ -19,6 +19,9 @@ names = {"sep-fused-tma0": (1, 1, 1, 0), "sep-fused-tma1": (1, 1, 1, 1), "sep-fu
          "sep-fused-direct": (1, 0, 1), "2d-tma": (0, 1, 0), "2d-direct": (0, 0, 0),
          "sep-unfused-tma": (1, 1, 0), "sep-unfused-direct": (1, 0, 0)}
 names["sep-fused-tma"] = names["sep-fused-tma0"]
+for cfg in range(8):                       # every fused TMA configuration, both store paths
+    names["sep-fused-tma%d" % cfg] = (1, 1, 1, cfg)
+    names["sep-fused-tma%ds8" % cfg] = (1, 1, 1, cfg, 1)
 H = W = a.size
 x = torch.rand((H, W), device="cuda")
 out = torch.empty((H - a.k + 1, W - a.k + 1), device="cuda")
