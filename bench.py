@@ -177,26 +177,24 @@ class ClockSampler:
 
 # --------------------------------------------------------------------------------------------
 class CleanFlush:
-    """The L2 flush between timed passes when the working set fits in L2: write a 2 x L2 scratch
-    buffer, then read a second 2 x L2 buffer, so the pass starts from an L2 of clean, unrelated
-    lines (a write alone leaves ~L2-size of dirty lines whose write-back the next pass would pay,
-    profiles/r02_flush_study.txt)."""
+    """The L2 flush between timed passes when the working set fits in L2: sepconv_l2_flush, which
+    writes a 2 x L2 buffer and then reads a second 2 x L2 buffer, so the pass starts from an L2
+    of clean, unrelated lines (a write alone leaves ~L2-size of dirty lines whose write-back the
+    next pass would pay, profiles/r02_flush_study.txt).  The tuner times its candidates after the
+    same flush, so its picks and this bench see the same conditions."""
 
     def __init__(self, torch, dev):
-        l2 = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
-        self.torch = torch
-        self.w = torch.empty(2 * l2 // 4, dtype=torch.float32, device=dev)
-        self.r = torch.zeros(2 * l2 // 4, dtype=torch.float32, device=dev)
-        self.sink = torch.empty((), dtype=torch.float32, device=dev)
+        from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc
+        self.sc = sc
+        self.stream = torch.cuda.current_stream(dev)
         for i in range(3):                       # first-call costs stay out of any timing
             self(i)
 
     def __call__(self, i=0):
-        self.w.fill_(float(i))
-        self.torch.sum(self.r, dim=0, out=self.sink)
+        self.sc.l2_flush(self.stream)
 
-    LABEL = ("L2 flushed before every step (write 2 x L2, then read another 2 x L2 so L2 holds clean unrelated "
-             "lines); step time = [events around steps x (flush + step)] - [mean of events around steps x flush "
+    LABEL = ("L2 flushed before every step (sepconv_l2_flush: write 2 x L2, then read another 2 x L2 so L2 holds "
+             "clean unrelated lines); step time = [events around steps x (flush + step)] - [mean of events around steps x flush "
              "before and after], / steps, after a spin-up of 20 flushes")
 
 

@@ -573,6 +573,43 @@ const char *sepconv_last_error(void) { return t_last_error.c_str(); }
 
 uint64_t sepconv_launch_count(void) { return g_launches.load(); }
 
+// The clean L2 flush of DESIGN.md R25, shared by the tuner's timing and bench.py: library-owned
+// scratch of 2 x L2 written, then a second 2 x L2 read, per device (allocated on first use).
+// Not counted by sepconv_launch_count (it is measurement hygiene, not SeparableConvolution).
+sepconv_status_t sepconv_l2_flush(sepconv_stream_t stream) {
+    clear_error();
+    int dev = -1;
+    SC_CUDA(cudaGetDevice(&dev));
+    struct Scratch {
+        float *w = nullptr, *r = nullptr, *sink = nullptr;
+        size_t n = 0;
+    };
+    static std::mutex mu;
+    static std::map<int, Scratch> all;
+    Scratch sc;
+    {
+        std::lock_guard<std::mutex> lock(mu);
+        auto it = all.find(dev);
+        if (it == all.end()) {
+            int l2 = 0;
+            SC_CUDA(cudaDeviceGetAttribute(&l2, cudaDevAttrL2CacheSize, dev));
+            Scratch n;
+            n.n = static_cast<size_t>(l2) / 2;                // floats in 2 x L2 bytes
+            SC_CUDA(cudaMalloc(&n.w, n.n * 4));
+            SC_CUDA(cudaMalloc(&n.r, n.n * 4));
+            SC_CUDA(cudaMalloc(&n.sink, 16));
+            SC_CUDA(cudaMemset(n.r, 0, n.n * 4));
+            SC_CUDA(cudaDeviceSynchronize());
+            it = all.emplace(dev, n).first;
+        }
+        sc = it->second;
+    }
+    cudaStream_t st = static_cast<cudaStream_t>(stream);
+    SC_CUDA(launch_l2_flush(sc.w, static_cast<long long>(sc.n), st));
+    SC_CUDA(launch_l2_clean(sc.r, static_cast<long long>(sc.n), sc.sink, st));
+    return SEPCONV_OK;
+}
+
 static sepconv_status_t validate_desc(const sepconv_plan_desc_t *d) {
     if (!d) return fail(SEPCONV_E_INVALID, "descriptor is NULL");
     if (d->k > SEPCONV_MAX_K) return fail(SEPCONV_E_UNSUPPORTED, "K=%d exceeds SEPCONV_MAX_K=%d", d->k, SEPCONV_MAX_K);

@@ -244,7 +244,7 @@ std::string cache_path_of(const sepconv_tune_opts_t *opts) {
 struct Bench {
     sepconv_plan_t plan = nullptr;
     Geometry g{};
-    float *din = nullptr, *dout = nullptr, *wflush = nullptr, *rflush = nullptr, *sink = nullptr;
+    float *din = nullptr, *dout = nullptr;
     size_t flush_floats = 0;
     bool need_flush = false;
     cudaStream_t st = nullptr;
@@ -261,15 +261,12 @@ struct Bench {
         if ((e = cudaMalloc(&din, in_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(in)");
         if ((e = cudaMalloc(&dout, out_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(out)");
         if (need_flush) {
-            if ((e = cudaMalloc(&wflush, flush_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(flush)");
-            if ((e = cudaMalloc(&rflush, flush_floats * 4)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(flush)");
-            if ((e = cudaMalloc(&sink, 16)) != cudaSuccess) return cuda_fail(e, "tune: cudaMalloc(sink)");
+            sepconv_status_t fs = sepconv_l2_flush(nullptr);   // allocates the shared scratch once
+            if (fs != SEPCONV_OK) return fs;
         }
         if ((e = cudaStreamCreateWithFlags(&st, cudaStreamNonBlocking)) != cudaSuccess) return cuda_fail(e, "tune: stream");
         if ((e = cudaEventCreate(&e0)) != cudaSuccess || (e = cudaEventCreate(&e1)) != cudaSuccess)
             return cuda_fail(e, "tune: events");
-        if (need_flush && (e = cudaMemsetAsync(rflush, 0, flush_floats * 4, st)) != cudaSuccess)
-            return cuda_fail(e, "tune: memset");
         launch_fill_pattern(din, static_cast<long long>(in_floats), 1234u, st);
         g = plan_geometry(p);
         kern.resize(p->k);
@@ -282,16 +279,13 @@ struct Bench {
     }
     ~Bench() {
         if (st) cudaStreamSynchronize(st);
-        for (float *b : {din, dout, wflush, rflush, sink})
+        for (float *b : {din, dout})
             if (b) cudaFree(b);
         if (e0) cudaEventDestroy(e0);
         if (e1) cudaEventDestroy(e1);
         if (st) cudaStreamDestroy(st);
     }
-    void flush() {
-        launch_l2_flush(wflush, static_cast<long long>(flush_floats), st);
-        launch_l2_clean(rflush, static_cast<long long>(flush_floats), sink, st);
-    }
+    void flush() { sepconv_l2_flush(st); }   // the same flush bench.py uses
     // event time of n iterations of body, in us per iteration
     sepconv_status_t batch(int n, const std::function<sepconv_status_t()> &body, double *us) {
         cudaEventRecord(e0, st);

@@ -885,6 +885,12 @@ sepconv_status_t sor_tune(sor_plan_t plan, int iters_hint, int reps, int *varian
         if (status != SEPCONV_OK) break;
         std::sort(times, times + R);
         const float med = times[R / 2];
+        if (const char *log = std::getenv("SEPCONV_TUNE_LOG"))    // diagnostics: every candidate's time
+            if (FILE *f = std::fopen(log, "a")) {
+                std::fprintf(f, "sor %lldx%lld depth %d seg_div %d: %.4f ms\n", (long long)plan->n, (long long)plan->m,
+                             d, div, med);
+                std::fclose(f);
+            }
         if (med < best * 0.99f) {
             best = med;
             best_v = d == 0 ? SOR_HALF : SOR_WAVE;

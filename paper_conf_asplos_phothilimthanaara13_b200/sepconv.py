@@ -174,6 +174,7 @@ def lib() -> ctypes.CDLL:
             "sepconv_last_error": (ctypes.c_char_p, []),
             "sepconv_version": (ctypes.c_char_p, []),
             "sepconv_launch_count": (ctypes.c_uint64, []),
+            "sepconv_l2_flush": (I, [P]),
         }
         for name, (res, args) in sig.items():
             fn = getattr(L, name)
@@ -187,6 +188,11 @@ def lib() -> ctypes.CDLL:
 def _check(st: int, where: str):
     if st != 0:
         raise SepconvError(st, where, (lib().sepconv_last_error() or b"").decode())
+
+
+def l2_flush(stream=None):
+    """sepconv_l2_flush: the clean L2 flush the tuner and bench.py time passes after."""
+    _check(lib().sepconv_l2_flush(_stream(stream)), "sepconv_l2_flush")
 
 
 def version() -> str:
@@ -205,7 +211,7 @@ def exported_symbols():
             "sepconv_num_candidates", "sepconv_get_candidate", "sepconv_band", "sepconv_nccl_unique_id",
             "sepconv_comm_init", "sepconv_run_band", "sepconv_band_trace", "sepconv_band_timeline",
             "sepconv_status_str", "sepconv_last_error",
-            "sepconv_version", "sepconv_launch_count"]
+            "sepconv_version", "sepconv_launch_count", "sepconv_l2_flush"]
 
 
 def _variant(v) -> int:
