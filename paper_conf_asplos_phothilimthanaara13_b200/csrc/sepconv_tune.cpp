@@ -16,7 +16,8 @@
 // traffic and not for write-backs of lines an unrelated kernel dirtied -- and the pass time is
 // the event time of n x (flush + pass) minus that of n x (flush), because single events tick
 // in 2.048 us steps on this system (profiles/r02_flush_study.txt); larger working sets time n
-// back-to-back passes.  The result is the fastest of three such batches (one-sided noise).
+// back-to-back passes.  The result is the fastest of three such batches (one-sided noise), or
+// for flushed differences their median (two-sided noise: the flush's own variance).
 //
 // sepconv_tune_selector(K): the exhaustive tuner at up to 12 square sizes, equal neighbouring
 // picks merged, each cutoff between different picks placed by timing both at the geometric
@@ -301,7 +302,7 @@ struct Bench {
         *us = ms * 1000.0 / n;
         return SEPCONV_OK;
     }
-    // the pass time of candidate c: the fastest of three batches of n (see the file comment)
+    // the pass time of candidate c from three batches of n (see the file comment)
     sepconv_status_t time(const Candidate &c, int n, float *out_us) {
         if (c.algo == SEPCONV_SEPARABLE && !c.fused) {
             sepconv_status_t s = ensure_buf(plan);
@@ -328,10 +329,12 @@ struct Bench {
                 if ((s = batch(n, pass, &t[b])) != SEPCONV_OK) return s;
             }
         }
-        // the fastest batch: the noise is one-sided (a transient clock, power or memory-system
-        // slowdown only adds time), and a median of three still let a 5% slowdown of one
-        // candidate's batches decide a pick (profiles/r02_tune_log.txt)
-        *out_us = static_cast<float>(std::min(t[0], std::min(t[1], t[2])));
+        // back-to-back batches: the fastest -- the noise is one-sided (a transient clock, power
+        // or memory-system slowdown only adds time), and a median of three still let a 5%
+        // slowdown of one candidate's batches decide a pick (profiles/r02_tune_log.txt).
+        // Flushed differences: the median -- the flush's own variance makes their noise two-sided
+        std::sort(t, t + 3);
+        *out_us = static_cast<float>(need_flush ? t[1] : t[0]);
         return SEPCONV_OK;
     }
 };
@@ -432,7 +435,7 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
     for (size_t ci = 0; ci < cs.size(); ++ci)
         if ((status = b.time(cs[ci], reps, &med[ci])) != SEPCONV_OK) return status;
     // finalists -- up to four candidates within 8% of the fastest -- are timed twice more in
-    // interleaved rounds and keep the fastest of their measurements: one sequential pass over
+    // interleaved rounds and keep the fastest (flushed: the median) of their measurements: one sequential pass over
     // the candidates picked a configuration 8% slower than the runner-up on 16384^2 / K=13 (a
     // transient during the runner-up's batches; profiles/r02_interleave.txt, r02_tune_log.txt)
     {
@@ -447,7 +450,11 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
             for (int round = 0; round < 2; ++round)
                 for (size_t f = 0; f < fin.size(); ++f)
                     if ((status = b.time(cs[fin[f]], reps, round ? &t2[f] : &t1[f])) != SEPCONV_OK) return status;
-            for (size_t f = 0; f < fin.size(); ++f) med[fin[f]] = std::min(med[fin[f]], std::min(t1[f], t2[f]));
+            for (size_t f = 0; f < fin.size(); ++f) {
+                float v[3] = {med[fin[f]], t1[f], t2[f]};
+                std::sort(v, v + 3);
+                med[fin[f]] = b.need_flush ? v[1] : v[0];      // as in Bench::time
+            }
         }
     }
 

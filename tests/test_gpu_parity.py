@@ -255,9 +255,12 @@ def test_launch_count_increases():
     assert sc.launch_count() == before + 2
 
 
-# ---- full BASELINE size, the configuration bench.py times, sampled rows --------------------
+# ---- full BASELINE size, untuned plan (static default and 2D), sampled rows -----------------
 @pytest.mark.parametrize("K", [3, 5, 7, 9, 11, 13, 15, 17])
 def test_full_size_16384_sampled_rows(K, _big_image):
+    """The untuned plan at 16384^2 (AUTO = the static default, and 2D) on sampled rows plus the
+    [0, 1) range property; the tuned configurations bench.py times are compared with the
+    oracle on every output cell in tests/test_gpu_fullsize.py."""
     img, dev_in = _big_image
     H = W = 16384
     ho, wo = H - K + 1, W - K + 1
