@@ -265,6 +265,29 @@ def emit(d):
     print(json.dumps(d), flush=True)
 
 
+def l2_bytes_of(dev=None):
+    """The device's L2 size (the flush rule); 126 MiB (B200) when no device is visible."""
+    try:
+        import torch
+        if torch.cuda.is_available():
+            return torch.cuda.get_device_properties(dev or 0).L2_cache_size or 126 * 2 ** 20
+    except Exception:
+        pass
+    return 126 * 2 ** 20
+
+
+def image_config(args, world, H, W, N_img, widths, seed, flush):
+    """The image / batch workload's `config`, identical for the CUDA arm and the reference arm."""
+    return {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
+                         if args.workload == "image" else f"{N_img} x {H}x{W} float32 images, width 11"),
+            "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
+            "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
+            "l2": (CleanFlush.LABEL.replace("step", "pass") + "; per width; ms_per_step = sum over widths")
+            if flush else "inputs larger than L2 (no flush)",
+            "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
+                            else f"images sharded x{world}" if world > 1 else "1 GPU")}
+
+
 # --------------------------------------------------------------------------------------------
 def run_reference(args):
     """--impl reference: the oracle (the paper's definition in plain C, double) on host cores."""
@@ -295,11 +318,10 @@ def run_reference(args):
         times.append(last["seconds"])
     value = statistics.median(vals)
     # the same workload string and keys as the CUDA arm's line (the oracle times a sample of it)
-    cfg = {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
-                        if args.workload == "image" else f"64 x {H}x{W} float32 images, width 11"),
-           "image": [H, W], "images": 1 if args.workload == "image" else 64, "widths": widths,
-           "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed, "sample": last["sample"],
-           "parallelism": "host cores (oracle)"}
+    # the CUDA arm's config, key for key (the oracle times a bounded sample of it: cpu_baseline.sample)
+    N_img = 1 if args.workload == "image" else 64
+    cfg = image_config(args, world, H, W, N_img, widths, seed,
+                       8 * H * W * N_img // max(world, 1) <= 2 * l2_bytes_of())
     emit({"impl": "reference", "metric": METRIC, "value": value, "unit": "Mpixels/s",
           "n_gpus": world if world > 1 else args.gpus,
           "steps": args.steps, "warmup": args.warmup, "ms_per_step": statistics.median(times) * 1e3,
@@ -373,10 +395,10 @@ def main():
         return run_dry(args)
     if args.workload == "poisson":
         import bench_poisson
-        return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed))
+        return bench_poisson.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed), l2_bytes_of())
     if args.workload == "blackscholes":
         import bench_bs
-        return bench_bs.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed))
+        return bench_bs.run(args, peaks, dist_env, ClockSampler, emit, (CleanFlush, time_flushed), l2_bytes_of())
     if args.impl == "reference":
         return run_reference(args)
 
@@ -649,14 +671,7 @@ def main():
             cpu["single_thread"] = {"value": one["value"], "unit": "Mpixels/s", "cores": 1, "sample": one["sample"]}
 
     if rank == 0:
-        cfg = {"workload": (f"{H}x{W} float32 image, kernel widths {','.join(map(str, widths))}, one pass per width"
-                            if args.workload == "image" else f"{N_img} x {H}x{W} float32 images, width 11"),
-               "image": [H, W], "images": N_img, "widths": widths, "variant": args.variant + " (tuned per width)",
-               "kernel": "normalised binomial C(K-1,i)/2^(K-1)", "seed": seed,
-               "l2": (CleanFlush.LABEL.replace("step", "pass") + "; per width; ms_per_step = sum over widths")
-               if flush else "inputs larger than L2 (no flush)",
-               "parallelism": (f"row bands x{world}, NCCL halo send/recv" if world > 1 and args.workload == "image"
-                               else f"images sharded x{world}" if world > 1 else "1 GPU")}
+        cfg = image_config(args, world, H, W, N_img, widths, seed, flush)
         emit({"metric": METRIC, "value": value, "unit": "Mpixels/s", "n_gpus": world, "steps": args.steps,
               "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": cfg,

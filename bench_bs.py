@@ -38,7 +38,14 @@ def _oracle_sample(target_s: float):
             "sample": f"{reps} x {n} options (oracle_black_scholes, double, one thread), {el:.1f} s"}
 
 
-def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
+def bs_config(n, world, flush, flush_label):
+    """The workload's `config`, identical for the CUDA arm and the reference arm."""
+    return {"workload": f"Black-Scholes, {n} float32 options per GPU (r={synth.BS_RATE}, v={synth.BS_VOL})",
+            "options": n, "l2": flush_label if flush else "inputs larger than L2 (no flush)",
+            "parallelism": f"options sharded x{world}" if world > 1 else "1 GPU"}
+
+
+def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None, l2_bytes=126 * 2 ** 20):
     world, rank, local = dist_env()
     if args.impl == "reference":
         if rank != 0:
@@ -53,9 +60,8 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
               "n_gpus": world if world > 1 else args.gpus,
               "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "weak",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-              "config": {"workload": (f"Black-Scholes, {args.options} float32 options per GPU "
-                                      f"(r={synth.BS_RATE}, v={synth.BS_VOL})"),
-                         "options": args.options, "sample": last["sample"], "parallelism": "host core (oracle)"},
+              # the CUDA arm's config, key for key (the oracle times a sample: cpu_baseline.sample)
+              "config": bs_config(args.options, world, 20 * args.options <= 2 * l2_bytes, flushing[0].LABEL),
               "cpu_baseline": {"value": v, "unit": "Moptions/s", "cores": 1, "kind": "oracle", "sample": last["sample"]},
               "e2e": {"value": v, "unit": "Moptions/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}})
         return 0
@@ -147,9 +153,7 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
         emit({"metric": METRIC, "value": value, "unit": "Moptions/s", "n_gpus": world, "steps": args.steps,
               "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
               "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-              "config": {"workload": f"Black-Scholes, {n} float32 options per GPU (r={r}, v={v})",
-                         "options": n, "l2": CleanFlush.LABEL if flush else "inputs larger than L2 (no flush)",
-                         "parallelism": f"options sharded x{world}" if world > 1 else "1 GPU"},
+              "config": bs_config(n, world, flush, CleanFlush.LABEL),
               "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
               "clocks": clk.summary()})
     if dist:

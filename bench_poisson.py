@@ -39,7 +39,15 @@ def _oracle_sample(target_s: float):
             "sample": f"{n}x{n} grid, {iters} red-black iterations in double (oracle_sor_rb, one thread), {t:.1f} s"}
 
 
-def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
+def sor_config(n, iters, world, flush, flush_label):
+    """The workload's `config`, identical for the CUDA arm and the reference arm."""
+    return {"workload": f"Poisson2D red-black SOR, {n}x{n} float32 grid, {iters} iterations per step",
+            "grid": [n, n], "iters_per_step": iters, "omega": synth.omega_opt(n, n),
+            "l2": (flush_label + "; the iterations of a step reuse L2") if flush else "grid larger than L2 (no flush)",
+            "parallelism": f"row bands x{world}" if world > 1 else "1 GPU"}
+
+
+def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None, l2_bytes=126 * 2 ** 20):
     if args.impl == "reference":
         world, rank, _ = dist_env()
         if rank != 0:
@@ -55,10 +63,9 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
               "n_gpus": world if world > 1 else args.gpus,
               "steps": args.steps, "warmup": args.warmup, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-              "config": {"workload": (f"Poisson2D red-black SOR, {args.size}x{args.size} float32 grid, "
-                                      f"{args.sor_iters} iterations per step"),
-                         "grid": [args.size, args.size], "iters_per_step": args.sor_iters,
-                         "sample": last["sample"], "parallelism": "host core (oracle)"},
+              # the CUDA arm's config, key for key (the oracle times a sample: cpu_baseline.sample)
+              "config": sor_config(args.size, args.sor_iters, world,
+                                   6 * args.size * args.size * 4 // max(world, 1) <= 2 * l2_bytes, flushing[0].LABEL),
               "cpu_baseline": {"value": v, "unit": "Mcell-it/s", "cores": 1, "kind": "oracle", "sample": last["sample"]},
               "e2e": {"value": v, "unit": "Mcell-it/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}})
         return 0
@@ -196,13 +203,9 @@ def run(args, peaks_fn, dist_env, ClockSampler, emit, flushing=None):
         emit({"metric": METRIC, "value": value, "unit": "Mcell-it/s", "n_gpus": world, "steps": args.steps,
               "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
               "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-              "config": {"workload": f"Poisson2D red-black SOR, {n}x{n} float32 grid, {iters} iterations per step",
-                         "grid": [n, n], "iters_per_step": iters, "omega": omega,
-                         "variant": "auto (tuned): " + ("half" if variant_id == sor.SOR_HALF else f"wave depth {depth}"),
-                         "l2": (CleanFlush.LABEL + "; the iterations of a step reuse L2") if flush
-                         else "grid larger than L2 (no flush)",
-                         "parallelism": (f"row bands x{world}, {2 * depth}-row ghost exchange per pass (NCCL)"
-                                         if world > 1 else "1 GPU")},
+              "config": sor_config(n, iters, world, flush, CleanFlush.LABEL),
+              "variant": "auto (tuned): " + ("half" if variant_id == sor.SOR_HALF else f"wave depth {depth}"),
+              "exchange": f"{2 * depth}-row ghost exchange per pass (NCCL)" if world > 1 else None,
               "gcell_it_s": value / 1e3, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
               "gpu_launches": int(launches), "launches_per_pass": launches_per, "clocks": clk.summary()})
     p.close()

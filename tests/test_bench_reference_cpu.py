@@ -29,6 +29,24 @@ def test_reference_arm_image_line():
     cb = d["cpu_baseline"]
     assert cb["kind"] == "oracle" and cb["cores"] >= 1 and cb["value"] == d["value"] and cb["sample"]
     assert d["e2e"] == {"value": d["value"], "unit": "Mpixels/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}
+    # the CUDA arm's config key for key (the driver compares the two arms' configs)
+    import argparse
+    import bench
+    args = argparse.Namespace(workload="image", variant="auto")
+    assert d["config"] == bench.image_config(args, 1, 96, 96, 1, [3, 5], d["config"]["seed"],
+                                             8 * 96 * 96 <= 2 * bench.l2_bytes_of())
+
+
+def test_reference_arm_poisson_and_black_scholes_lines():
+    import bench_bs
+    import bench_poisson
+    from bench import CleanFlush
+    p = run_bench("--workload", "poisson", "--size", "64", "--sor-iters", "4")
+    assert p["impl"] == "reference" and p["unit"] == "Mcell-it/s" and p["value"] > 0
+    assert p["config"] == bench_poisson.sor_config(64, 4, 1, True, CleanFlush.LABEL)
+    b = run_bench("--workload", "blackscholes", "--options", "1000")
+    assert b["impl"] == "reference" and b["unit"] == "Moptions/s" and b["value"] > 0
+    assert b["config"] == bench_bs.bs_config(1000, 1, True, CleanFlush.LABEL)
 
 
 def test_reference_arm_other_ranks_exit_quietly():
