@@ -376,11 +376,20 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
     const double sigma = 0.5 * std::log(2.0);
     Candidate parent = best;
     float parent_us = best_us;
-    for (int m = 0; m < mutations; ++m) {
-        const double u = rng.uniform();
+    const double parts0 = parts;
+    for (int m = 0; m < mutations + 2; ++m) {
         double np = parts, ng = grid;
-        if (u < 2.0 / 3.0) np = parts * std::exp(sigma * rng.normal());
-        if (u >= 1.0 / 3.0) ng = grid * std::exp(sigma * rng.normal());
+        if (m < 2) {
+            // seeded members of the initial population: two and three rounds of the model's
+            // items over every slot (more, shorter segments average out per-SM speed
+            // differences: 16384^2 / K=17 -7.5%, profiles/r02_sched_check.txt)
+            np = parts0 * (m + 2);
+            ng = static_cast<double>(slots);
+        } else {
+            const double u = rng.uniform();
+            if (u < 2.0 / 3.0) np = parts * std::exp(sigma * rng.normal());
+            if (u >= 1.0 / 3.0) ng = grid * std::exp(sigma * rng.normal());
+        }
         np = std::min<double>(std::max(1.0, std::round(np)), rows);
         ng = std::min(std::max(1.0, std::round(ng)), static_cast<double>(slots));
         Candidate child = parent;
@@ -438,9 +447,10 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
     // interleaved rounds and keep the fastest (flushed: the median) of their measurements: one sequential pass over
     // the candidates picked a configuration 8% slower than the runner-up on 16384^2 / K=13 (a
     // transient during the runner-up's batches; profiles/r02_interleave.txt, r02_tune_log.txt)
+    std::vector<size_t> finalists;
     {
         const float fastest = *std::min_element(med.begin(), med.end());
-        std::vector<size_t> fin;
+        std::vector<size_t> &fin = finalists;
         for (size_t i = 0; i < cs.size(); ++i)
             if (med[i] >= 0 && med[i] <= fastest * 1.08f) fin.push_back(i);
         std::sort(fin.begin(), fin.end(), [&](size_t a, size_t c) { return med[a] < med[c]; });
@@ -489,10 +499,40 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
         win[s] = cs[bi[s]];
         us[s] = med[bi[s]];
     }
-    // the paper's evolutionary refinement of size-like tunables, on AUTO's winner
-    if ((status = mutate_schedule(b, win[2], us[2], mutations, seed, reps)) != SEPCONV_OK) return status;
+    // the paper's evolutionary refinement of size-like tunables, on each single-kernel finalist
+    // (up to three): a configuration that loses under the model's schedule can win under its
+    // own best schedule (16384^2 / K=17: cfg 4 with 27 parts beats cfg 3, which gains nothing)
+    if (mutations > 0) {
+        std::vector<size_t> pool;
+        for (size_t i : finalists)
+            if (passes(cs[i]) == 1 && pool.size() < 3) pool.push_back(i);
+        if (pool.empty()) pool.push_back(bi[2]);
+        std::vector<std::pair<Candidate, float>> out;
+        for (size_t i : pool) {
+            Candidate c = cs[i];
+            float t = med[i];
+            if ((status = mutate_schedule(b, c, t, mutations, seed, reps)) != SEPCONV_OK) return status;
+            out.emplace_back(c, t);
+        }
+        // fastest wins; within 1% of it the lower candidate index (R17)
+        float tmin = out[0].second;
+        for (auto &o : out) tmin = std::min(tmin, o.second);
+        size_t pick = SIZE_MAX, k_pick = 0;
+        for (size_t k = 0; k < out.size(); ++k)
+            if (out[k].second <= tmin * 1.01f && (pick == SIZE_MAX || pool[k] < pick)) {
+                pick = pool[k];
+                k_pick = k;
+            }
+        const Candidate pick_c = out[k_pick].first;
+        const float pick_t = out[k_pick].second;
+        if (pick_t < us[2] || pick == bi[2]) {
+            win[2] = pick_c;
+            us[2] = pick_t;
+            bi[2] = pick;
+        }
+    }
     const int aslot = win[2].algo == SEPCONV_2D ? 0 : 1;
-    if (bi[aslot] == bi[2]) {
+    if (bi[aslot] == bi[2] || us[2] < us[aslot]) {
         win[aslot] = win[2];
         us[aslot] = us[2];
     }
