@@ -42,3 +42,22 @@ for g in range(2):
     q.run_band(band, synth.binomial_kernel(K), out, "auto")
     torch.cuda.synchronize()
     print("ok run_band", g, flush=True)
+
+# round 2: schedule overrides (the mutation search's tunables), the replay fast path and the
+# clean L2 flush
+h, w, K = 1200, 2300, 13
+img = torch.from_numpy(synth.uniform_image(h, w, seed=3)).cuda()
+out = torch.empty((h - K + 1, w - K + 1), device="cuda")
+p = sc.Plan(h, w, K)
+for cfg in range(6):
+    for parts, grid in ((1, 1), (7, 20), (300, 0)):
+        p.run_choice(img, synth.binomial_kernel(K), out,
+                     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, sched_parts=parts, sched_grid=grid))
+        torch.cuda.synchronize()
+    print("ok overrides cfg", cfg, flush=True)
+run = p.bind(img, synth.binomial_kernel(K), out, "separable")
+for _ in range(3):
+    run()
+sc.l2_flush()
+torch.cuda.synchronize()
+print("ok replay + l2_flush", flush=True)
