@@ -106,35 +106,6 @@ __device__ __forceinline__ void tma_refill_elected(bool go, void *dst, const CUt
         : "memory");
 }
 
-// CTA-shared stage refill (CS configurations): NB boxes of BXW columns side by side, each into its
-// own 128-byte aligned block of BLK floats, one expect_tx for all of them; issued by warp 0's
-// elected lane under a predicate (no branch).
-template <int NB, int BXW, int BLK>
-__device__ __forceinline__ void tma_refill_cta(bool go, float *dst, const CUtensorMap *map, uint64_t *bar,
-                                               uint32_t bytes, int c0, int c1, int c2) {
-    asm volatile(
-        "{\n\t.reg .pred e, g, q;\n\t"
-        "elect.sync _|e, 0xffffffff;\n\t"
-        "setp.ne.u32 g, %0, 0;\n\t"
-        "and.pred q, e, g;\n\t"
-        "@q fence.proxy.async.shared::cta;\n\t"
-        "@q mbarrier.arrive.expect_tx.shared::cta.b64 _, [%1], %2;\n\t}" ::"r"(static_cast<uint32_t>(go)),
-        "r"(smem_u32(bar)), "r"(bytes)
-        : "memory");
-#pragma unroll
-    for (int b = 0; b < NB; ++b)
-        asm volatile(
-            "{\n\t.reg .pred e, g, q;\n\t"
-            "elect.sync _|e, 0xffffffff;\n\t"
-            "setp.ne.u32 g, %6, 0;\n\t"
-            "and.pred q, e, g;\n\t"
-            "@q cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes "
-            "[%0], [%1, {%3, %4, %5}], [%2];\n\t}" ::"r"(smem_u32(dst + b * BLK)),
-            "l"(reinterpret_cast<uint64_t>(map)), "r"(smem_u32(bar)), "r"(c0 + b * BXW), "r"(c1), "r"(c2),
-            "r"(static_cast<uint32_t>(go))
-            : "memory");
-}
-
 __device__ __forceinline__ void prefetch_tmap(const CUtensorMap *map) {
     asm volatile("prefetch.tensormap [%0];" ::"l"(reinterpret_cast<uint64_t>(map)) : "memory");
 }
@@ -395,7 +366,7 @@ struct SegmentIter {
 // One CTA = NW independent warps over NW adjacent 128-column strips; the CTA's
 // share of the (image, CTA-strip, row) space is contiguous, split evenly over
 // the grid so the row granularity is 1 and no CTA idles at the end.
-template <int K, int OP, int MAP, int NW, int SR_, int NS_, int F2, int SM = 1, int LOCK = 0, int CS = 0>
+template <int K, int OP, int MAP, int NW, int SR_, int NS_, int F2, int SM = 1, int LOCK = 0>
 __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel(const __grid_constant__ StreamParams p) {
     constexpr bool TMA = MAP == MAP_TMA;
     constexpr bool HALO = OP != OP_COLS;
@@ -412,53 +383,21 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     static_assert(BW <= 256, "TMA box width");
     static_assert(BW == box_width(K, HALO), "box width");
     static_assert(!RING || SR % K == 0, "ring period must divide the stage");
-    // CS: one CTA-wide stage of SR rows x (NW*128 + halo) columns, shared by the warps (the
-    // halo columns are loaded once per CTA, not once per warp), as NB boxes of BXW columns in
-    // 128-byte aligned blocks of BLK floats; refilled by warp 0 after a CTA barrier
-    constexpr int CW = stream_cta_cols(K, OP, NW);
-    constexpr int NB = (CW + 255) / 256;
-    constexpr int BXW = ((CW + NB - 1) / NB + 3) & ~3;
-    constexpr int BLK = (SR * BXW + 31) & ~31;
-    constexpr int CSTAGE = NB * BLK;
-    constexpr int CBYTES = NB * SR * BXW * 4;
-    static_assert(!CS || (TMA && LOCK && RING), "CTA-shared stages need TMA, the CTA lockstep barrier and OP_SEP/COLS");
-    static_assert(!TMA || CS || NW * NS * (STAGE * 4 + 8) <= kSmemPerCta, "shared memory per CTA");
-    static_assert(!CS || NS * (CSTAGE * 4 + 8) <= kSmemPerCta, "shared memory per CTA");
+    static_assert(!TMA || NW * NS * (STAGE * 4 + 8) <= kSmemPerCta, "shared memory per CTA");
 
     extern __shared__ __align__(128) float smem[];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    float *wsm = smem + (TMA && !CS ? warp * NS * STAGE : 0);
-    uint64_t *wbar = CS ? reinterpret_cast<uint64_t *>(smem + NS * CSTAGE)
-                        : reinterpret_cast<uint64_t *>(smem + NW * NS * STAGE) + warp * NS;
-    // CS: this thread's window float4 v lives at coff[v] + row * BXW of a stage
-    int coff[XV];
-    if constexpr (CS) {
-#pragma unroll
-        for (int v = 0; v < XV; ++v) {
-            const int col = warp * kWarpCols + lane * V + 4 * v;
-            const int b = col / BXW;
-            coff[v] = b * BLK + (col - b * BXW);
-        }
-    }
+    float *wsm = smem + (TMA ? warp * NS * STAGE : 0);
+    uint64_t *wbar = reinterpret_cast<uint64_t *>(smem + NW * NS * STAGE) + warp * NS;
 
     if constexpr (TMA) {
-        if constexpr (CS) {
-            if (threadIdx.x == 0) {
-                prefetch_tmap(&p.tmap);
+        if (lane == 0) {
+            if (warp == 0) prefetch_tmap(&p.tmap);
 #pragma unroll
-                for (int s = 0; s < NS; ++s) mbar_init(&wbar[s], 1);
-                fence_barrier_init();
-            }
-            __syncthreads();
-        } else {
-            if (lane == 0) {
-                if (warp == 0) prefetch_tmap(&p.tmap);
-#pragma unroll
-                for (int s = 0; s < NS; ++s) mbar_init(&wbar[s], 1);
-                fence_barrier_init();
-            }
-            __syncwarp();
+            for (int s = 0; s < NS; ++s) mbar_init(&wbar[s], 1);
+            fence_barrier_init();
         }
+        __syncwarp();
     }
 
     SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg, p.win_rows, p.extra);
@@ -474,12 +413,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             __syncthreads();
         }
         const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
-        if (wcol >= p.out_cols) {
-            // CS: the stages' barrier phases are shared, so an idle warp keeps its chunk count
-            // in step with the warps that consume this segment
-            if constexpr (CS) kc += (nrows + (RING ? K - 1 : 0) + SR - 1) / SR;
-            continue;
-        }
+        if (wcol >= p.out_cols) continue;
         // warps of this strip that have columns (named-barrier thread count for LOCK)
         const int lock_threads = 32 * min(NW, (p.out_cols - s * (NW * kWarpCols) + kWarpCols - 1) / kWarpCols);
         (void)lock_threads;
@@ -493,22 +427,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         OutCursor oc;
         oc.init(out_rows - (RING ? static_cast<long long>(K - 1) * p.ld_out : 0LL), p.ld_out, c, p.out_cols);
 
-        if constexpr (TMA && CS) {
-            // the per-segment CTA barrier above ordered every warp's reads of the previous
-            // segment before these async-proxy writes; warp 0 loads the whole CTA strip
-            if (warp == 0 && lane == 0) {
-                fence_proxy_async_smem();
-                const int npro = nchunks < NS ? nchunks : NS;
-                const int ccol = s * (NW * kWarpCols);
-                for (int ch = 0; ch < npro; ++ch) {
-                    const int st = (kc + ch) % NS;
-                    mbar_arrive_expect_tx(&wbar[st], CBYTES);
-                    for (int b = 0; b < NB; ++b)
-                        tma_load_3d(smem + st * CSTAGE + b * BLK, &p.tmap, &wbar[st], ccol + b * BXW,
-                                    in_row0 + ch * SR, n);
-                }
-            }
-        } else if constexpr (TMA) {
+        if constexpr (TMA) {
             __syncwarp();                                      // every lane is past the previous segment's reads
             if (lane == 0) {
                 fence_proxy_async_smem();                      // ... which precede these async-proxy writes
@@ -533,19 +452,13 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
 
         for (int ch = 0; ch < nchunks; ++ch, ++kc) {
             const int st = kc % NS;
-            const float *stage = CS ? smem + st * CSTAGE : wsm + st * STAGE;
+            const float *stage = wsm + st * STAGE;
             if constexpr (TMA) mbar_wait(&wbar[st], (kc / NS) & 1);
 #pragma unroll
             for (int pr = 0; pr < SR; ++pr) {
                 const int t = ch * SR + pr;                    // step = input row - in_row0
                 float x[XV * 4];
-                if constexpr (TMA && CS) {
-#pragma unroll
-                    for (int v = 0; v < XV; ++v) {
-                        const float4 tt = ld_shared4(stage + coff[v] + pr * BXW);
-                        x[4 * v + 0] = tt.x; x[4 * v + 1] = tt.y; x[4 * v + 2] = tt.z; x[4 * v + 3] = tt.w;
-                    }
-                } else if constexpr (TMA) {
+                if constexpr (TMA) {
 #pragma unroll
                     for (int v = 0; v < XV; ++v) {
                         const float4 tt = ld_shared4(stage + pr * BW + lane * V + 4 * v);
@@ -635,12 +548,8 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                 } else {
                     __syncwarp();
                 }
-                if constexpr (CS)
-                    tma_refill_cta<NB, BXW, BLK>(warp == 0 && ch + NS < nchunks, smem + st * CSTAGE, &p.tmap,
-                                                 &wbar[st], CBYTES, s * (NW * kWarpCols), in_row0 + (ch + NS) * SR, n);
-                else
-                    tma_refill_elected(ch + NS < nchunks, wsm + st * STAGE, &p.tmap, &wbar[st], BOX_BYTES, wcol,
-                                       in_row0 + (ch + NS) * SR, n);
+                tma_refill_elected(ch + NS < nchunks, wsm + st * STAGE, &p.tmap, &wbar[st], BOX_BYTES, wcol,
+                                   in_row0 + (ch + NS) * SR, n);
             }
         }
         };
@@ -654,14 +563,10 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     }
 }
 
-template <int K, int OP, int MAP, int NW, int SR, int NS, int F2, int CS = 0>
+template <int K, int OP, int MAP, int NW, int SR, int NS, int F2>
 constexpr size_t stream_smem_bytes() {
-    if (MAP != MAP_TMA) return 0;
-    if (CS) {
-        const int cw = stream_cta_cols(K, OP, NW), nb = (cw + 255) / 256, bxw = ((cw + nb - 1) / nb + 3) & ~3;
-        return static_cast<size_t>(NS) * nb * ((SR * bxw + 31) & ~31) * 4 + NS * 8;
-    }
-    return static_cast<size_t>(NW) * NS * ((SR * stream_bw(K, OP) + 31) & ~31) * 4 + NW * NS * 8;
+    return MAP == MAP_TMA ? static_cast<size_t>(NW) * NS * ((SR * stream_bw(K, OP) + 31) & ~31) * 4 + NW * NS * 8
+                          : 0;
 }
 
 // The kernel for (K, OP, variant) with the geometry of stream_geom (sepconv_params.h).

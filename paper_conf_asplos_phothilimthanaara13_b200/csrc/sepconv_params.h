@@ -90,10 +90,6 @@ constexpr int kSmemPerCta = 232448 - 1024;     // opt-in limit minus headroom
 
 SEPCONV_HD constexpr int stream_bw(int K, int op) { return 32 * 4 + (op != OP_COLS ? (((K - 1) + 3) & ~3) : 0); }
 SEPCONV_HD constexpr int stage_floats(int sr, int bw) { return (sr * bw + 31) & ~31; }   // 128-byte aligned
-// columns one CTA-shared stage row holds (CS configurations): the CTA's strip plus one halo
-SEPCONV_HD constexpr int stream_cta_cols(int K, int op, int nw) {
-    return nw * 32 * 4 + (op != OP_COLS ? (((K - 1) + 3) & ~3) : 0);
-}
 SEPCONV_HD constexpr int ns_fit(int nw, int sr, int bw) { return kSmemPerCta / (nw * (stage_floats(sr, bw) * 4 + 8)); }
 SEPCONV_HD constexpr int clampi(int v, int lo, int hi) { return v < lo ? lo : (v > hi ? hi : v); }
 
