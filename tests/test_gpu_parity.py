@@ -349,6 +349,28 @@ def test_repeated_calls_refresh_weights_and_choices():
     check(img, kb, out.cpu().numpy())
 
 
+def test_l2_flush_and_tuner_without_mutation():
+    """sepconv_l2_flush is measurement hygiene: it launches no SeparableConvolution kernel (the
+    launch counter does not move) and leaves results untouched; a tune with the mutation search
+    off returns the model's schedule (no override), a tuned pick with it on is still one of the
+    candidates, and both match the oracle."""
+    h, w, K = 900, 1300, 7
+    img = synth.uniform_image(h, w, seed=12)
+    k = synth.binomial_kernel(K)
+    before = sc.launch_count()
+    for _ in range(3):
+        sc.l2_flush()
+    torch.cuda.synchronize()
+    assert sc.launch_count() == before
+    p = sc.Plan(h, w, K)
+    plain = p.tune(reps=3, force=True, mutations=-1)
+    assert plain.sched_parts == 0 and plain.sched_grid == 0 and plain.source == sc.SRC_TUNED
+    check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
+    mutated = p.tune(reps=3, force=True, mutations=6, seed=3)
+    assert mutated.base_name in {c.name for c in p.candidates()}
+    check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
+
+
 def test_band_timeline_orders_the_phases():
     """sepconv_band_trace / sepconv_band_timeline (the overlap evidence of SURVEY 8(e)): on a
     middle band in external-halo mode the interior kernel, the (empty) exchange and the tail
