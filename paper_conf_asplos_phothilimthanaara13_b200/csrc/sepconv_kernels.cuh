@@ -490,8 +490,9 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                             b[e + 1] = bb.y;
                         }
                     } else if constexpr (F2 == 3 && K >= 2) {
-                        // (exploration) two independent chains over even / odd taps, halving the
-                        // row pass's dependent-FMA depth: b = (sum_even) + (sum_odd)
+                        // exploration only (tools/explore_mid.cu; no product configuration uses
+                        // it: it changes the summation order R6): two independent chains over
+                        // even / odd taps, halving the row pass's dependent-FMA depth
 #pragma unroll
                         for (int e = 0; e < V; ++e) {
                             float b0 = p.k[0] * x[e], b1 = p.k[1] * x[e + 1];
