@@ -402,9 +402,16 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
 
     SegmentIter seg(p.total, p.rows, p.nstrips, p.parts, p.nimg, p.win_rows, p.extra);
     uint32_t kc = 0;                                           // chunks consumed by this warp
+#ifdef SEPCONV_CTA_TRACE
+    unsigned long long t_start = 0, nseg = 0;
+    if (threadIdx.x == 0) asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_start));
+#endif
 
     int n, s, q0, nrows;
     while (seg.next(n, s, q0, nrows)) {
+#ifdef SEPCONV_CTA_TRACE
+        ++nseg;
+#endif
         if constexpr (TMA && LOCK) {
             // the lockstep barrier's thread count depends on the strip: a warp must not reach
             // the next segment's barriers while another still uses this one's (a CTA whose
@@ -562,6 +569,19 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         if (wcol + kWarpCols <= p.out_cols && p.store8 >= SM) run_chunks(std::integral_constant<int, SMF>{});
         else run_chunks(std::integral_constant<int, 0>{});
     }
+#ifdef SEPCONV_CTA_TRACE
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned long long t_end;
+        unsigned smid;
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_end));
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+        p.trace[4 * blockIdx.x + 0] = t_start;
+        p.trace[4 * blockIdx.x + 1] = t_end;
+        p.trace[4 * blockIdx.x + 2] = smid;
+        p.trace[4 * blockIdx.x + 3] = nseg;
+    }
+#endif
 }
 
 template <int K, int OP, int MAP, int NW, int SR, int NS, int F2>

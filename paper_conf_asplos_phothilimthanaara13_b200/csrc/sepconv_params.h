@@ -45,6 +45,10 @@ struct alignas(64) StreamParams {
     int extra;                   // parts < 0: CTAs sharing the last (short) window
     float k[kMaxK];
     float2 k2[kMaxK];            // {k_i, k_i}: the same weights as packed-FP32 operands
+#ifdef SEPCONV_CTA_TRACE
+    unsigned long long *trace;   // exploration builds only (tools/explore_mid.cu): per CTA
+                                 // {start ns, end ns, SM id, segments}
+#endif
 };
 
 struct alignas(64) Conv2DParams {
