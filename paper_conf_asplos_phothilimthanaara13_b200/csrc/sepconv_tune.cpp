@@ -15,9 +15,9 @@
 // flush -- a write of 2 x L2 then a read of another 2 x L2, so the pass pays for its own
 // traffic and not for write-backs of lines an unrelated kernel dirtied -- and the pass time is
 // the event time of n x (flush + pass) minus that of n x (flush), because single events tick
-// in 2.048 us steps on this system (profiles/r02_flush_study.txt); larger working sets time
-// back-to-back passes in batches of >= ~15 ms after a warm-up batch (sustained clocks and power).
-// The result is the median of three such batches.
+// in 2.048 us steps on this system (profiles/r02_flush_study.txt); larger working sets time n
+// back-to-back passes.  The result is the fastest of three such batches (one-sided noise), or
+// for flushed differences their median (two-sided noise: the flush's own variance).
 //
 // sepconv_tune_selector(K): the exhaustive tuner at up to 12 square sizes, equal neighbouring
 // picks merged, each cutoff between different picks placed by timing both at the geometric
@@ -320,32 +320,21 @@ struct Bench {
         sepconv_status_t s = pass();                              // warm-up (first-launch costs)
         if (s != SEPCONV_OK) return s;
         double t[3];
-        int nb = n;
-        if (!need_flush) {
-            // back-to-back passes are timed in batches of >= ~15 ms after a warm-up batch of the
-            // same length, so that clocks and the power controller reach the state a sustained
-            // stream of passes runs in: short bursts favoured the FMA-heaviest configuration at
-            // 16384^2 / K=17, which then ran 5% slower under bench.py's sustained load with the
-            // power cap active (profiles/r02_driver_bench.json)
-            double probe = 0;
-            if ((s = batch(n, pass, &probe)) != SEPCONV_OK) return s;
-            if (probe > 0 && probe < 1500.0) nb = std::min(200, std::max(n, static_cast<int>(std::ceil(15000.0 / probe))));
-            double warm = 0;
-            if ((s = batch(nb, pass, &warm)) != SEPCONV_OK) return s;
-        }
         for (int b = 0; b < 3; ++b) {
             if (need_flush) {
                 double tf = 0, tfp = 0;
                 if ((s = batch(n, fl, &tf)) != SEPCONV_OK || (s = batch(n, flpass, &tfp)) != SEPCONV_OK) return s;
                 t[b] = std::max(0.05, tfp - tf);
             } else {
-                if ((s = batch(nb, pass, &t[b])) != SEPCONV_OK) return s;
+                if ((s = batch(n, pass, &t[b])) != SEPCONV_OK) return s;
             }
         }
-        // the median of three batches (the finalists' interleaved re-timing then absorbs a
-        // transient slowdown of one candidate's batches, profiles/r02_tune_log.txt)
+        // back-to-back batches: the fastest -- the noise is one-sided (a transient clock, power
+        // or memory-system slowdown only adds time), and a median of three still let a 5%
+        // slowdown of one candidate's batches decide a pick (profiles/r02_tune_log.txt).
+        // Flushed differences: the median -- the flush's own variance makes their noise two-sided
         std::sort(t, t + 3);
-        *out_us = static_cast<float>(t[1]);
+        *out_us = static_cast<float>(need_flush ? t[1] : t[0]);
         return SEPCONV_OK;
     }
 };
@@ -455,7 +444,7 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
     for (size_t ci = 0; ci < cs.size(); ++ci)
         if ((status = b.time(cs[ci], reps, &med[ci])) != SEPCONV_OK) return status;
     // finalists -- up to four candidates within 8% of the fastest -- are timed twice more in
-    // interleaved rounds and keep the median of their three measurements: one sequential pass over
+    // interleaved rounds and keep the fastest (flushed: the median) of their measurements: one sequential pass over
     // the candidates picked a configuration 8% slower than the runner-up on 16384^2 / K=13 (a
     // transient during the runner-up's batches; profiles/r02_interleave.txt, r02_tune_log.txt)
     std::vector<size_t> finalists;
@@ -474,7 +463,7 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
             for (size_t f = 0; f < fin.size(); ++f) {
                 float v[3] = {med[fin[f]], t1[f], t2[f]};
                 std::sort(v, v + 3);
-                med[fin[f]] = v[1];
+                med[fin[f]] = b.need_flush ? v[1] : v[0];      // as in Bench::time
             }
         }
     }
