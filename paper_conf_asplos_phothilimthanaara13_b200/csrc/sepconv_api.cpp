@@ -293,14 +293,34 @@ static Sched schedule(const DeviceInfo &di, int occ, int nimg, int nstrips, int 
 // A tuner-mutated schedule (sepconv_choice_t.sched_parts / sched_grid) replaces the model's:
 // `parts` strided row partitions per (image, strip) over `grid` CTAs, both clamped to what the
 // geometry and the resident slots allow.  Any (parts, grid) is a valid SegmentIter schedule.
+static constexpr int kMaxClaims = 1 << 16;
+
 static Sched apply_override(const Sched &model, long long slots, int nimg, int nstrips, int rows, int parts,
-                            int grid) {
+                            int grid, int steal = 0, int warps = 1, int stage_rows = 1, int K = 1) {
     if (parts <= 0) return model;
     const long long p = std::max(1, std::min(parts, rows));
     const long long items = static_cast<long long>(nimg) * nstrips * p;
     long long g = grid > 0 ? grid : slots;
     g = std::max<long long>(1, std::min(std::min(g, slots), items));
-    return Sched{static_cast<int>(g), static_cast<int>(p), 0, 0};
+    Sched sc{static_cast<int>(g), static_cast<int>(p), 0, 0};
+    // work stealing: one claim word per (segment, warp), stage counts in 16 bits
+    const long long max_stages = ((rows + p - 1) / p + K - 1) / stage_rows + 2;
+    if (steal > 0 && steal < 100 && items * warps <= kMaxClaims && max_stages < 65535) sc.steal = steal;
+    return sc;
+}
+
+// the kernels that carry the work-stealing code (sepconv_kernels.cuh: fused TMA, free-running
+// warps, at most 8 per CTA)
+static bool steal_ok(int op, bool tma, int map, int K, int warps) {
+    return op == OP_SEP && tma && warps <= 8 && !stream_geom(K, OP_SEP, map).lock;
+}
+
+static sepconv_status_t ensure_claims(sepconv_plan_t plan) {
+    if (plan->claims) return SEPCONV_OK;
+    SC_CUDA(cudaMalloc(&plan->claims, kMaxClaims * sizeof(unsigned long long)));
+    SC_CUDA(cudaMemset(plan->claims, 0, kMaxClaims * sizeof(unsigned long long)));
+    SC_CUDA(cudaDeviceSynchronize());          // zeroed before any stream's first stealing launch
+    return SEPCONV_OK;
 }
 
 // One streaming pass (ROWS, COLS or SEP) over geometry g.
@@ -308,7 +328,7 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
                                          long long ld_in, long long in_img, int in_cols, float *out,
                                          long long ld_out, long long out_img, int out_cols, int rows_total,
                                          const float *kernel, bool want_tma, int cfg, int store_path,
-                                         cudaStream_t st, int ov_parts = 0, int ov_grid = 0,
+                                         cudaStream_t st, int ov_parts = 0, int ov_grid = 0, int ov_steal = 0,
                                          Sched *query = nullptr, long long *query_slots = nullptr,
                                          sepconv_plan_s::Replay *record = nullptr) {
     const int K = g.K;
@@ -354,7 +374,9 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     }
     const long long slots = static_cast<long long>(plan->dev.sms) * occ;
     const Sched sc = apply_override(schedule(plan->dev, occ, g.nimg, p.nstrips, rows_total, K), slots, g.nimg,
-                                    p.nstrips, rows_total, ov_parts, ov_grid);
+                                    p.nstrips, rows_total, ov_parts, ov_grid,
+                                    steal_ok(op, tma, map, K, ki.threads / 32) ? ov_steal : 0, ki.threads / 32,
+                                    std::max(1, ki.stage_rows), K);
     if (query) {                                               // candidate_sched: report, do not launch
         *query = sc;
         if (query_slots) *query_slots = slots;
@@ -364,6 +386,14 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     p.parts = sc.parts;
     p.win_rows = sc.win_rows;
     p.extra = sc.extra;
+    if (sc.steal > 0) {
+        s = ensure_claims(plan);
+        if (s != SEPCONV_OK) return s;
+        p.steal = sc.steal;
+        p.claims = plan->claims;
+        p.epoch = ++plan->epoch;
+        if (p.epoch == 0) p.epoch = ++plan->epoch;             // 0 is the words' initial value
+    }
     cudaError_t e = stream_launch(op, map, K, smode, p, sc.grid, st);
     if (e != cudaSuccess) return cuda_fail(e, "stream kernel launch");
     g_launches.fetch_add(1, std::memory_order_relaxed);
@@ -452,11 +482,11 @@ sepconv_status_t launch_candidate(sepconv_plan_t plan, const Geometry &g, const 
     // a schedule override was tuned for the plan's whole geometry; bands and host-pipeline
     // chunks (other row counts) use the model
     const bool whole = g.row_begin == 0 && g.rows == plan->ho && g.nimg == plan->n;
-    const int ovp = whole ? c.sched_parts : 0, ovg = whole ? c.sched_grid : 0;
+    const int ovp = whole ? c.sched_parts : 0, ovg = whole ? c.sched_grid : 0, ovs = whole ? c.sched_steal : 0;
     if (c.algo == SEPCONV_2D) return launch_2d(plan, g, in, out, kernel, tma, st, ovp, ovg);
     if (c.fused)
         return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img,
-                                g.out_cols, g.rows, kernel, tma, c.config, c.store, st, ovp, ovg);
+                                g.out_cols, g.rows, kernel, tma, c.config, c.store, st, ovp, ovg, ovs);
     // Choice 2 as the paper writes it: ConvolveRows into buffer, then ConvolveColumns.
     // The buffer holds the rows this launch's output rows need: [row_begin, row_begin + rows + K - 1).
     if (!buf) return fail(SEPCONV_E_INVALID, "unfused separable needs a workspace");
@@ -498,7 +528,8 @@ sepconv_status_t candidate_sched(sepconv_plan_t plan, const Geometry &g, const C
         return launch_2d(plan, g, in, out, k.data(), tma, nullptr, c.sched_parts, c.sched_grid, sc, slots);
     if (!c.fused) return fail(SEPCONV_E_INVALID, "candidate_sched: the unfused pair has two schedules");
     return launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img, g.out_cols,
-                            g.rows, k.data(), tma, c.config, c.store, nullptr, c.sched_parts, c.sched_grid, sc, slots);
+                            g.rows, k.data(), tma, c.config, c.store, nullptr, c.sched_parts, c.sched_grid,
+                            c.sched_steal, sc, slots);
 }
 
 Candidate from_choice(const sepconv_choice_t &c) {
@@ -506,6 +537,7 @@ Candidate from_choice(const sepconv_choice_t &c) {
                 c.store_path};
     r.sched_parts = c.sched_parts;
     r.sched_grid = c.sched_grid;
+    r.sched_steal = c.sched_steal;
     return r;
 }
 
@@ -523,6 +555,7 @@ sepconv_choice_t to_choice(const Candidate &c, int K, int source) {
                         : 1;
     o.sched_parts = c.sched_parts;
     o.sched_grid = c.sched_grid;
+    o.sched_steal = c.sched_steal;
     o.source = source;
     return o;
 }
@@ -691,6 +724,7 @@ void sepconv_destroy(sepconv_plan_t plan) {
     if (plan->last_work) cudaEventDestroy(plan->last_work);
     for (auto &e : plan->tev)
         if (e) cudaEventDestroy(e);
+    if (plan->claims) cudaFree(plan->claims);
     delete plan;
 }
 
@@ -724,6 +758,7 @@ static sepconv_status_t check_choice(const sepconv_choice_t *c) {
     if (c->store_path < 0 || c->store_path > 1) return fail(SEPCONV_E_INVALID, "choice.store_path must be 0 or 1");
     if (c->sched_parts < 0 || c->sched_grid < 0)
         return fail(SEPCONV_E_INVALID, "choice.sched_parts / sched_grid must be >= 0");
+    if (c->sched_steal < 0 || c->sched_steal > 99) return fail(SEPCONV_E_INVALID, "choice.sched_steal must be in [0, 99]");
     return SEPCONV_OK;
 }
 
@@ -749,10 +784,14 @@ static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const
     const int mode = sched_mode();
     if (r.valid && r.in == in && r.out == out && r.algo == c.algo && r.mapping == c.mapping && r.fused == c.fused &&
         r.config == c.config && r.store == c.store && r.sched_parts == c.sched_parts &&
-        r.sched_grid == c.sched_grid && r.sched_mode == mode) {
+        r.sched_grid == c.sched_grid && r.sched_steal == c.sched_steal && r.sched_mode == mode) {
         for (int i = 0; i < plan->k; ++i) {
             r.p.k[i] = kernel[i];
             r.p.k2[i] = make_float2(kernel[i], kernel[i]);
+        }
+        if (r.p.steal > 0) {                                   // a fresh claim epoch per launch
+            r.p.epoch = ++plan->epoch;
+            if (r.p.epoch == 0) r.p.epoch = ++plan->epoch;
         }
         if (r.p.total <= 0) return SEPCONV_OK;
         cudaError_t e = stream_launch(r.op, r.map, plan->k, r.smode, r.p, r.grid, st);
@@ -763,7 +802,7 @@ static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const
     r.valid = false;
     s = launch_stream_op(plan, OP_SEP, g, in, g.ld_in, g.in_img, g.in_cols, out, g.ld_out, g.out_img, g.out_cols,
                          g.rows, kernel, c.mapping == SEPCONV_MAP_TMA, c.config, c.store, st, c.sched_parts,
-                         c.sched_grid, nullptr, nullptr, &r);
+                         c.sched_grid, c.sched_steal, nullptr, nullptr, &r);
     if (s == SEPCONV_OK && r.valid) {
         r.in = in;
         r.out = out;
@@ -774,6 +813,7 @@ static sepconv_status_t run_resolved(sepconv_plan_t plan, const float *in, const
         r.store = c.store;
         r.sched_parts = c.sched_parts;
         r.sched_grid = c.sched_grid;
+        r.sched_steal = c.sched_steal;
         r.sched_mode = mode;
     }
     return s;

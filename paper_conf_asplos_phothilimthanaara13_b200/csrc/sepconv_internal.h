@@ -53,12 +53,14 @@ struct Candidate {
     int store;     // 0: 16-byte store path when every output row allows it, 1: always the 8-byte path
     int sched_parts = 0;   // work-schedule override (sepconv_choice_t.sched_parts): 0 = model
     int sched_grid = 0;    // CTAs of the override (0 = every resident slot)
+    int sched_steal = 0;   // work stealing between warps: minimum stages a victim must have left (0 = off)
 };
 
 // The work schedule a launch uses (SegmentIter, sepconv_kernels.cuh): grid CTAs; parts > 0
 // strided row partitions, 0 contiguous, -q the window schedule (win_rows, extra).
 struct Sched {
     int grid, parts, win_rows, extra;
+    int steal = 0;         // work-stealing threshold (strided schedule; 0 = off)
 };
 
 struct TensorMapCache {
@@ -104,12 +106,17 @@ struct sepconv_plan_s {
         bool valid = false;
         const float *in = nullptr;
         float *out = nullptr;
-        int algo = -1, mapping = -1, fused = -1, config = -1, store = -1, sched_parts = 0, sched_grid = 0;
+        int algo = -1, mapping = -1, fused = -1, config = -1, store = -1, sched_parts = 0, sched_grid = 0,
+            sched_steal = 0;
         int sched_mode = 0;                 // $SEPCONV_SCHED at record time
         int op = 0, map = 0, smode = 0, grid = 0;
         sepconv::StreamParams p;
     } replay;
     cudaEvent_t last_work = nullptr;
+
+    // work stealing (sched_steal): a launch counter tags the claim words of each launch
+    unsigned epoch = 0;
+    unsigned long long *claims = nullptr;   // kMaxClaims words, zeroed at allocation
 
     // NCCL (row bands)
     void *comm = nullptr;

@@ -362,6 +362,81 @@ struct SegmentIter {
     }
 };
 
+// ---- work stealing between warps ---------------------------------------------------------
+// With p.steal > 0 (strided schedule), warp w of segment item d owns the claim word
+// claims[d * NW + w] = epoch:32 | front:16 | end:16, in TMA stages ("chunks") of that warp's
+// column strip.  The owner claims its stages one at a time from the front (an atomic add one
+// stage ahead of use, so the latency hides behind a stage of arithmetic); a warp that has run
+// out of work takes half of the largest unclaimed remainder from the back by compare-and-swap
+// and computes it as an ordinary segment (K-1 warm-up rows).  A thief always leaves the owner
+// its next stage, so the owner stops exactly where the thief starts: every output row is
+// computed by one warp, with the same arithmetic as any other schedule.  Words of an earlier
+// launch carry an older epoch and are ignored.
+__device__ __forceinline__ unsigned long long claim_word(unsigned epoch, int front, int end) {
+    return (static_cast<unsigned long long>(epoch) << 32) | (static_cast<unsigned long long>(front) << 16) |
+           static_cast<unsigned long long>(end);
+}
+
+// segment of item d under the strided schedule (SegmentIter, parts > 0)
+__device__ __forceinline__ void strided_item(long long d, int rows, int nstrips, int parts, int &n, int &s, int &q0,
+                                             int &nrows) {
+    s = static_cast<int>(d % nstrips);
+    const long long t = d / nstrips;
+    const int j = static_cast<int>(t % parts);
+    n = static_cast<int>(t / parts);
+    q0 = static_cast<int>(static_cast<long long>(rows) * j / parts);
+    nrows = static_cast<int>(static_cast<long long>(rows) * (j + 1) / parts) - q0;
+}
+
+// Called by all 32 lanes of a warp with no work left: steals half of the largest unclaimed
+// remainder (at least p.steal stages) of any warp of this launch.  Returns the stolen rows as a
+// segment of warp slot wslot, or false when nothing is worth stealing.
+template <int K, int SR, int NW>
+__device__ bool steal_stages(const StreamParams &p, int lane, int &n, int &s, int &wslot, int &q0, int &nrows) {
+    const long long nwords = static_cast<long long>(p.nimg) * p.nstrips * p.parts * NW;
+    for (int attempt = 0; attempt < 64; ++attempt) {
+        int best_rem = 0;
+        long long best_v = -1;
+        unsigned long long best_w = 0;
+        for (long long v = lane; v < nwords; v += 32) {
+            const unsigned long long w = *reinterpret_cast<volatile unsigned long long *>(p.claims + v);
+            if (static_cast<unsigned>(w >> 32) != p.epoch) continue;
+            const int rem = static_cast<int>(w & 0xffff) - static_cast<int>((w >> 16) & 0xffff);
+            if (rem > best_rem) {
+                best_rem = rem;
+                best_v = v;
+                best_w = w;
+            }
+        }
+#pragma unroll
+        for (int o = 16; o; o >>= 1) {                          // warp argmax (ties: lower index)
+            const int r2 = __shfl_xor_sync(0xffffffffu, best_rem, o);
+            const long long v2 = __shfl_xor_sync(0xffffffffu, best_v, o);
+            const unsigned long long w2 = __shfl_xor_sync(0xffffffffu, best_w, o);
+            if (r2 > best_rem || (r2 == best_rem && v2 < best_v)) {
+                best_rem = r2;
+                best_v = v2;
+                best_w = w2;
+            }
+        }
+        if (best_rem < p.steal || best_rem < 2) return false;
+        const int f = static_cast<int>((best_w >> 16) & 0xffff), e = static_cast<int>(best_w & 0xffff);
+        const int e_new = e - (e - f) / 2;                       // >= f + 1: the owner keeps its next stage
+        int won = 0;
+        if (lane == 0)
+            won = atomicCAS(p.claims + best_v, best_w, (best_w & ~0xffffull) | static_cast<unsigned>(e_new)) == best_w;
+        if (!__shfl_sync(0xffffffffu, won, 0)) continue;        // the word moved: look again
+        wslot = static_cast<int>(best_v % NW);
+        strided_item(best_v / NW, p.rows, p.nstrips, p.parts, n, s, q0, nrows);
+        const int r0 = e_new * SR - (K - 1);                      // output rows of stages [e_new, e)
+        const int r1 = min(e * SR - (K - 1), nrows);
+        q0 += r0;
+        nrows = r1 - r0;
+        return true;
+    }
+    return false;
+}
+
 // ---- the streaming kernel -----------------------------------------------------------
 // One CTA = NW independent warps over NW adjacent 128-column strips; the CTA's
 // share of the (image, CTA-strip, row) space is contiguous, split evenly over
@@ -407,8 +482,25 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     if (threadIdx.x == 0) asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_start));
 #endif
 
+    // work stealing between warps: free-running warps only (lockstep CTAs share barriers; the
+    // 16-warp CTAs' 128-register budget has no room for the claim state)
+    constexpr bool STEAL = TMA && RING && !LOCK && NW <= 8;
+    const bool steal_on = STEAL && p.steal > 0 && p.parts > 0;
+    bool thief = false;
     int n, s, q0, nrows;
-    while (seg.next(n, s, q0, nrows)) {
+    for (;;) {
+        int wslot = warp;                                      // column slot (a thief takes its victim's)
+        unsigned long long *word = nullptr;                    // this warp-segment's claim word (owner)
+        if (!thief) {
+            if (seg.next(n, s, q0, nrows)) {
+                if (steal_on) word = p.claims + (seg.item - gridDim.x) * NW + warp;
+            } else if (steal_on) {
+                thief = true;
+            } else {
+                break;
+            }
+        }
+        if (thief && !steal_stages<K, SR, NW>(p, lane, n, s, wslot, q0, nrows)) break;
 #ifdef SEPCONV_CTA_TRACE
         ++nseg;
 #endif
@@ -419,7 +511,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             // window schedule would otherwise mix counts on barrier 1)
             __syncthreads();
         }
-        const int wcol = s * (NW * kWarpCols) + warp * kWarpCols;   // warp's first column
+        const int wcol = s * (NW * kWarpCols) + wslot * kWarpCols;  // warp's first column
         if (wcol >= p.out_cols) continue;
         // warps of this strip that have columns (named-barrier thread count for LOCK)
         const int lock_threads = 32 * min(NW, (p.out_cols - s * (NW * kWarpCols) + kWarpCols - 1) / kWarpCols);
@@ -439,6 +531,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
             if (lane == 0) {
                 fence_proxy_async_smem();                      // ... which precede these async-proxy writes
                 const int npro = nchunks < NS ? nchunks : NS;
+                if (word) atomicExch(word, claim_word(p.epoch, npro, nchunks));   // open for thieves
                 for (int ch = 0; ch < npro; ++ch) {
                     const int st = (kc + ch) % NS;
                     mbar_arrive_expect_tx(&wbar[st], BOX_BYTES);
@@ -457,7 +550,12 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
 #pragma unroll
             for (int e = 0; e < V; ++e) acc[a][e] = 0.f;
 
-        for (int ch = 0; ch < nchunks; ++ch, ++kc) {
+        // stealing: stages [0, limit) are this warp's; the claim of stage `next` is issued one
+        // refill ahead of its use (pend, lane 0)
+        int limit = nchunks;
+        unsigned long long pend = 0;
+        if (STEAL && word != nullptr && lane == 0 && NS < nchunks) pend = atomicAdd(word, 1ull << 16);
+        for (int ch = 0; ch < limit; ++ch, ++kc) {
             const int st = kc % NS;
             const float *stage = wsm + st * STAGE;
             if constexpr (TMA) mbar_wait(&wbar[st], (kc / NS) & 1);
@@ -556,7 +654,17 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                 } else {
                     __syncwarp();
                 }
-                tma_refill_elected(ch + NS < nchunks, wsm + st * STAGE, &p.tmap, &wbar[st], BOX_BYTES, wcol,
+                bool go = ch + NS < limit;
+                if (STEAL && word != nullptr && go) {          // warp-uniform
+                    const unsigned long long r = __shfl_sync(0xffffffffu, pend, 0);
+                    if (((r >> 16) & 0xffff) < (r & 0xffff)) {  // stage ch + NS is ours
+                        if (lane == 0 && ch + NS + 1 < nchunks) pend = atomicAdd(word, 1ull << 16);
+                    } else {                                   // a thief has the rest
+                        limit = ch + NS;
+                        go = false;
+                    }
+                }
+                tma_refill_elected(go, wsm + st * STAGE, &p.tmap, &wbar[st], BOX_BYTES, wcol,
                                    in_row0 + (ch + NS) * SR, n);
             }
         }

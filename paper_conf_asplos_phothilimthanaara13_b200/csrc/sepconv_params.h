@@ -43,6 +43,11 @@ struct alignas(64) StreamParams {
     long long total;             // nimg * nstrips * rows (work units)
     int win_rows;                // parts < 0: rows of each of the q main windows
     int extra;                   // parts < 0: CTAs sharing the last (short) window
+    int steal;                   // work stealing between warps (strided schedule): a warp out of work
+                                 // takes half of another's unclaimed stages when at least this many
+                                 // remain (0 = off)
+    unsigned epoch;              // launch id the claim words are tagged with
+    unsigned long long *claims;  // claim word per (segment item, warp) (plan-owned)
     float k[kMaxK];
     float2 k2[kMaxK];            // {k_i, k_i}: the same weights as packed-FP32 operands
 #ifdef SEPCONV_CTA_TRACE

@@ -81,19 +81,28 @@ std::string selector_key(const DeviceInfo &d, int K) {
 // ---- the JSON-lines cache -------------------------------------------------------------------
 std::string choice_json(const sepconv_choice_t &c) {
     char b[200];
-    snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g,%d,%d]", (int)c.algo, c.mapping, c.fused, c.config,
-             c.store_path, c.warps, c.ctas_per_sm, c.median_us, c.sched_parts, c.sched_grid);
+    if (c.sched_steal)                                         // 11 fields only when stealing is on
+        snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g,%d,%d,%d]", (int)c.algo, c.mapping, c.fused, c.config,
+                 c.store_path, c.warps, c.ctas_per_sm, c.median_us, c.sched_parts, c.sched_grid, c.sched_steal);
+    else
+        snprintf(b, sizeof b, "[%d,%d,%d,%d,%d,%d,%d,%.9g,%d,%d]", (int)c.algo, c.mapping, c.fused, c.config,
+                 c.store_path, c.warps, c.ctas_per_sm, c.median_us, c.sched_parts, c.sched_grid);
     return b;
 }
 
 // parses one "[...]" choice at p; returns the position after it, or nullptr
 const char *parse_choice_at(const char *p, sepconv_choice_t *c) {
-    int algo, map, fused, config, store, warps, ctas, parts = 0, grid = 0, used = 0;
+    int algo, map, fused, config, store, warps, ctas, parts = 0, grid = 0, steal = 0, used = 0;
     float us;
     if (sscanf(p, "[%d,%d,%d,%d,%d,%d,%d,%f,%d,%d]%n", &algo, &map, &fused, &config, &store, &warps, &ctas, &us, &parts,
-               &grid, &used) != 10 || used == 0)
-        return nullptr;
+               &grid, &used) != 10 || used == 0) {
+        used = 0;
+        if (sscanf(p, "[%d,%d,%d,%d,%d,%d,%d,%f,%d,%d,%d]%n", &algo, &map, &fused, &config, &store, &warps, &ctas, &us,
+                   &parts, &grid, &steal, &used) != 11 || used == 0)
+            return nullptr;
+    }
     if (store < 0 || store > 1 || config < 0 || config >= kSepTmaConfigs || parts < 0 || grid < 0) return nullptr;
+    if (steal < 0 || steal > 99) return nullptr;
     if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return nullptr;
     std::memset(c, 0, sizeof *c);
     c->algo = static_cast<sepconv_variant_t>(algo);
@@ -106,6 +115,7 @@ const char *parse_choice_at(const char *p, sepconv_choice_t *c) {
     c->median_us = us;
     c->sched_parts = parts;
     c->sched_grid = grid;
+    c->sched_steal = steal;
     return p + used;
 }
 
@@ -362,7 +372,7 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
     Sched model;
     long long slots = 0;
     Candidate probe = best;
-    probe.sched_parts = probe.sched_grid = 0;
+    probe.sched_parts = probe.sched_grid = probe.sched_steal = 0;
     sepconv_status_t s = candidate_sched(b.plan, b.g, probe, &model, &slots);
     if (s != SEPCONV_OK) return s;
     const int rows = b.g.rows;
@@ -377,26 +387,46 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
     Candidate parent = best;
     float parent_us = best_us;
     const double parts0 = parts;
-    for (int m = 0; m < mutations + 2; ++m) {
+    // work stealing between warps (R27) is seeded on the configurations that carry it
+    // (fused TMA with free-running warps, at most 8 per CTA: cfg 2, 4, 5)
+    const bool stealing = best.algo == SEPCONV_SEPARABLE && best.fused && best.mapping == SEPCONV_MAP_TMA &&
+                          (best.config == 2 || best.config == 4 || best.config == 5);
+    const int nseeds = stealing ? 4 : 2;
+    int steal = best.sched_steal;
+    for (int m = 0; m < mutations + nseeds; ++m) {
         double np = parts, ng = grid;
+        int nst = steal;
         if (m < 2) {
             // seeded members of the initial population: two and three rounds of the model's
             // items over every slot (more, shorter segments average out per-SM speed
             // differences: 16384^2 / K=17 -7.5%, profiles/r02_sched_check.txt)
             np = parts0 * (m + 2);
             ng = static_cast<double>(slots);
+            nst = 0;
+        } else if (m < nseeds) {
+            // stealing on one and on two rounds of the model's items: warps that run out of
+            // work take half of the largest unclaimed remainder (profiles/r02_steal_sched.txt)
+            np = parts0 * (m - 1);
+            ng = static_cast<double>(slots);
+            nst = 4;
         } else {
             const double u = rng.uniform();
             if (u < 2.0 / 3.0) np = parts * std::exp(sigma * rng.normal());
             if (u >= 1.0 / 3.0) ng = grid * std::exp(sigma * rng.normal());
+            if (steal > 0 && rng.uniform() < 0.5)             // the stealing threshold, in stages
+                nst = static_cast<int>(std::lround(steal * std::exp(sigma * rng.normal())));
+            nst = steal > 0 ? std::min(std::max(nst, 2), 64) : 0;
         }
         np = std::min<double>(std::max(1.0, std::round(np)), rows);
         ng = std::min(std::max(1.0, std::round(ng)), static_cast<double>(slots));
         Candidate child = parent;
         child.sched_parts = static_cast<int>(np);
         child.sched_grid = static_cast<int>(ng);
+        child.sched_steal = nst;
         float us = 0.f;
         if ((s = b.time(child, reps, &us)) != SEPCONV_OK) return s;
+        const float parent_before = parent_us;
+        bool accepted = false;
         if (us < parent_us * 0.98f) {
             // a paired re-measurement (parent, child, parent, child) decides: batch-to-batch
             // drift of ~1-2% on 16384^2 otherwise admits children that are not faster
@@ -407,12 +437,22 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
             }
             const float p2 = std::min(tp[0], tp[1]), c2 = std::min(tc[0], tc[1]);
             if (c2 < p2 * 0.99f) {
+                accepted = true;
                 parent = child;
                 parent_us = c2;
                 parts = np;
                 grid = ng;
+                steal = nst;
             } else if (p2 < parent_us) {
                 parent_us = p2;
+            }
+        }
+        if (const char *log = std::getenv("SEPCONV_TUNE_LOG")) {   // diagnostics: every child
+            if (FILE *f = std::fopen(log, "a")) {
+                std::fprintf(f, "mutation k%d cfg%d s%d: child p%dg%dst%d %.2f us vs parent %.2f -> %s\n", b.g.K,
+                             child.config, child.store, child.sched_parts, child.sched_grid, child.sched_steal, us,
+                             parent_before, accepted ? "accepted" : "rejected");
+                std::fclose(f);
             }
         }
     }
@@ -510,12 +550,13 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
         us[s] = med[bi[s]];
     }
     // the paper's evolutionary refinement of size-like tunables, on each single-kernel finalist
-    // (up to three): a configuration that loses under the model's schedule can win under its
-    // own best schedule (16384^2 / K=17: cfg 4 with 27 parts beats cfg 3, which gains nothing)
+    // (up to four): a configuration that loses under the model's schedule can win under its
+    // own best schedule (16384^2 / K=17: cfg 4 with 27 parts beats cfg 3, which gains nothing;
+    // the fourth finalist is kept for configurations that only win with work stealing)
     if (mutations > 0) {
         std::vector<size_t> pool;
         for (size_t i : finalists)
-            if (passes(cs[i]) == 1 && pool.size() < 3) pool.push_back(i);
+            if (passes(cs[i]) == 1 && pool.size() < 4) pool.push_back(i);
         if (pool.empty()) pool.push_back(bi[2]);
         std::vector<std::pair<Candidate, float>> out;
         for (size_t i : pool) {
@@ -599,7 +640,7 @@ void sepconv_seed_from_cache(sepconv_plan_t plan) {
     if (!load_selector(env, selector_key(plan->dev, plan->k), &sel) || sel.k != plan->k) return;
     sepconv_choice_t pick;
     if (sepconv_select(&sel, plan->n * plan->h * plan->w, &pick) != SEPCONV_OK) return;
-    pick.sched_parts = pick.sched_grid = 0;                    // size-specific: not transferred
+    pick.sched_parts = pick.sched_grid = pick.sched_steal = 0;                    // size-specific: not transferred
     const int slot = pick.algo == SEPCONV_2D ? 0 : 1;
     for (int s = 0; s < 3; ++s) {
         // 2D / SEPARABLE requests keep their static defaults unless the selector picked that algorithm
@@ -722,7 +763,7 @@ sepconv_status_t sepconv_tune_selector(int K, int device, const int64_t *sides, 
         ++sel.m;
     }
     for (int i = 0; i < sel.m; ++i) {
-        sel.algos[i].sched_parts = sel.algos[i].sched_grid = 0;
+        sel.algos[i].sched_parts = sel.algos[i].sched_grid = sel.algos[i].sched_steal = 0;
         sel.algos[i].source = SEPCONV_SRC_SELECTOR;
     }
     const std::string path = cache_path_of(opts);

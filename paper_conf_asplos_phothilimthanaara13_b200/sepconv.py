@@ -50,7 +50,7 @@ class _Choice(ctypes.Structure):
                 ("config", ctypes.c_int), ("store_path", ctypes.c_int), ("warps", ctypes.c_int),
                 ("ctas_per_sm", ctypes.c_int),
                 ("median_us", ctypes.c_float), ("sched_parts", ctypes.c_int), ("sched_grid", ctypes.c_int),
-                ("source", ctypes.c_int)]
+                ("sched_steal", ctypes.c_int), ("source", ctypes.c_int)]
 
 
 class _TuneOpts(ctypes.Structure):
@@ -76,6 +76,7 @@ class Choice:
     sched_parts: int = 0          # tuned work-schedule override (0 = the library's model)
     sched_grid: int = 0
     source: int = SRC_EXPLICIT    # SRC_DEFAULT / SRC_TUNED / SRC_SELECTOR / SRC_EXPLICIT
+    sched_steal: int = 0          # work-stealing threshold in stages (0 = off); strided overrides only
 
     @property
     def base_name(self) -> str:
@@ -88,19 +89,21 @@ class Choice:
 
     @property
     def name(self) -> str:
-        return self.base_name + ("@p%dg%d" % (self.sched_parts, self.sched_grid) if self.sched_parts else "")
+        s = ("@p%dg%d" % (self.sched_parts, self.sched_grid)) if self.sched_parts else ""
+        return self.base_name + s + ("st%d" % self.sched_steal if self.sched_parts and self.sched_steal else "")
 
     def key(self):
-        return (self.algo, self.mapping, self.fused, self.config, self.store_path, self.sched_parts, self.sched_grid)
+        return (self.algo, self.mapping, self.fused, self.config, self.store_path, self.sched_parts, self.sched_grid,
+                self.sched_steal)
 
     def _c(self) -> _Choice:
         return _Choice(self.algo, self.mapping, self.fused, self.config, self.store_path, self.warps, self.ctas_per_sm,
-                       self.median_us, self.sched_parts, self.sched_grid, self.source)
+                       self.median_us, self.sched_parts, self.sched_grid, self.sched_steal, self.source)
 
     @staticmethod
     def _from(c: _Choice) -> "Choice":
         return Choice(c.algo, c.mapping, c.fused, c.config, c.store_path, c.warps, c.ctas_per_sm, float(c.median_us),
-                      c.sched_parts, c.sched_grid, c.source)
+                      c.sched_parts, c.sched_grid, c.source, c.sched_steal)
 
 
 @dataclass(frozen=True)

@@ -168,7 +168,7 @@ static void cache_fuzz() {
     const std::string gpu = std::string(prop.name) + "|" + std::to_string(prop.multiProcessorCount);
     const std::string good_plan = "{\"key\":\"" + gpu +
                                   "|1x300x200|k5|ld200,196\",\"2d\":[0,1,0,0,0,8,1,3.5,0,0],\"sep\":"
-                                  "[1,1,1,2,0,8,1,2.5,7,100],\"auto\":[1,1,1,2,0,8,1,2.5,7,100]}";
+                                  "[1,1,1,2,0,8,1,2.5,7,100],\"auto\":[1,1,1,2,0,8,1,2.5,7,100,85]}";
     const std::string good_sel = "{\"key\":\"sel:" + gpu +
                                  "|k5\",\"k\":5,\"m\":3,\"cutoffs\":[10000,90000],\"algos\":[[0,1,0,0,0,8,1,0,0,0],"
                                  "[1,1,1,1,0,8,1,0,0,0],[1,1,1,3,1,16,1,0,0,0]]}";
@@ -185,6 +185,7 @@ static void cache_fuzz() {
             sepconv_choice_t c;
             EXPECT(sepconv_get_choice(p, SEPCONV_AUTO, &c) == SEPCONV_OK);
             EXPECT(c.config >= 0 && c.config < 8 && c.sched_parts >= 0 && c.sched_grid >= 0);
+            EXPECT(c.sched_steal >= 0 && c.sched_steal <= 99);
             sepconv_destroy(p);
         }
     }
@@ -197,7 +198,11 @@ static void cache_fuzz() {
         if (sepconv_plan_ex(&d, &p) == SEPCONV_OK) {
             sepconv_choice_t c;
             sepconv_get_choice(p, SEPCONV_AUTO, &c);
-            EXPECT(c.source == SEPCONV_SRC_TUNED && c.config == 2 && c.sched_parts == 7 && c.sched_grid == 100);
+            EXPECT(c.source == SEPCONV_SRC_TUNED && c.config == 2 && c.sched_parts == 7 && c.sched_grid == 100 &&
+                   c.sched_steal == 85);
+            sepconv_choice_t sc;
+            sepconv_get_choice(p, SEPCONV_SEPARABLE, &sc);
+            EXPECT(sc.sched_parts == 7 && sc.sched_steal == 0);          // the 10-field form: no stealing
             sepconv_destroy(p);
         }
         sepconv_plan_desc_t d2{1, 250, 250, 5, 0, 0, -1};            // 62500 px: level 2 of 3

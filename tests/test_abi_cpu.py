@@ -186,3 +186,13 @@ def test_select_rejects_malformed_selectors(cutoffs, m):
     out = sc._Choice()
     import ctypes
     assert sc.lib().sepconv_select(ctypes.byref(s), 100, ctypes.byref(out)) == -1   # E_INVALID
+
+
+def test_choice_names_and_steal_field():
+    """The Python Choice mirrors sepconv_choice_t field for field (sched_steal included) and names
+    a schedule override as @p<parts>g<grid>[st<threshold>]."""
+    c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 4, sched_parts=18, sched_grid=148, sched_steal=4)
+    assert c.name == "sep-fused-tma4@p18g148st4"
+    assert sc.Choice._from(c._c()) == c
+    assert sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2, sched_steal=4).name == "sep-fused-tma2"
+    assert [f[0] for f in sc._Choice._fields_][-2:] == ["sched_steal", "source"]

@@ -477,6 +477,43 @@ def test_mutated_schedules_are_bitwise_equal_and_tuned_one_is_kept(tmp_path):
     check(img, k, run_gpu(img, k, variant="auto", plan=p)[0])
 
 
+@pytest.mark.parametrize("n,h,w,K,cfg,parts,grid", [
+    (1, 2048, 2048, 17, 2, 74, 0),     # 2 strips x 74 parts = 148 segments, one per CTA
+    (1, 2048, 2048, 17, 4, 70, 0),     # 140 segments on 148 slots
+    (1, 2048, 2048, 17, 5, 74, 0),     # 4-warp CTAs, 2 per SM: 4 strips x 74 = 296 segments
+    (1, 2048, 2048, 17, 2, 300, 148),  # 600 segments, ~4 per CTA
+    (1, 2048, 2048, 17, 2, 5, 7),      # few long segments: thieves split them repeatedly
+    (1, 2048, 2048, 17, 0, 74, 0),     # lockstep stages: stealing compiled out, override applies
+    (1, 2048, 2048, 17, 3, 148, 0),    # 16 warps: likewise
+    (3, 601, 700, 9, 2, 49, 0),        # a batch, ragged 700-column strip
+    (1, 1000, 3000, 5, 4, 9, 20),      # 3 strips, the last one ragged; K=5 (stage = 10 rows)
+    (1, 1000, 3000, 3, 5, 40, 0),      # K=3 (stage = 6 rows)
+])
+def test_work_stealing_bitwise(n, h, w, K, cfg, parts, grid):
+    """Work stealing between warps (sched_steal, R27) moves the unclaimed stages of a
+    warp's rows to whichever warp runs out of work first; it changes no pixel's arithmetic, so
+    every threshold gives the model schedule's bits, on repeated launches (a fresh claim epoch
+    each, through the replay fast path) that reuse the same claim words."""
+    img = synth.uniform_image(n * h, w, seed=31).reshape(n, h, w)
+    k = synth.random_kernel(K, seed=5, signed=True)
+    p = sc.Plan(h, w, K, n=n)
+    dev = torch.from_numpy(img).cuda()
+    ref = torch.empty((n, h - K + 1, w - K + 1), device="cuda")
+    p.run_choice(dev, k, ref, sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg))
+    torch.cuda.synchronize()
+    for i in range(n):
+        check(img[i], k, ref[i].cpu().numpy())
+    for steal in (1, 2, 4, 16, 99, 4):
+        c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, sched_parts=parts, sched_grid=grid,
+                      sched_steal=steal)
+        assert c.name.endswith("st%d" % steal)
+        for _ in range(3):
+            out = torch.full_like(ref, float("nan"))
+            p.run_choice(dev, k, out, c)
+            torch.cuda.synchronize()
+            assert torch.equal(out, ref), (steal, c.name)
+
+
 # ---- work schedules: the window schedule (every SM busy) equals the others bit for bit -----
 @pytest.mark.parametrize("choice", [CANDS[i] for i in (0, 2, 3, 4, 5, 7, 8, 10)],
                          ids=[IDS[i] for i in (0, 2, 3, 4, 5, 7, 8, 10)])

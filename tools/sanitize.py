@@ -55,6 +55,16 @@ for cfg in range(6):
                      sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, sched_parts=parts, sched_grid=grid))
         torch.cuda.synchronize()
     print("ok overrides cfg", cfg, flush=True)
+# work stealing between warps (claim words, the owners' stage claims, the thieves' scan and
+# compare-and-swap): one segment per CTA, several per CTA, and few long ones
+for cfg in (2, 4, 5):
+    for parts, grid in ((49, 0), (300, 0), (4, 9)):
+        for steal in (2, 8):
+            p.run_choice(img, synth.binomial_kernel(K), out,
+                         sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, sched_parts=parts, sched_grid=grid,
+                                   sched_steal=steal))
+            torch.cuda.synchronize()
+    print("ok work stealing cfg", cfg, flush=True)
 run = p.bind(img, synth.binomial_kernel(K), out, "separable")
 for _ in range(3):
     run()

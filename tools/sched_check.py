@@ -1,6 +1,7 @@
 """Times fused candidates with explicit work-schedule overrides on one plan (device-resident,
 back-to-back batches; clean-flushed batch differences when the working set fits in L2).
-    python tools/sched_check.py --size 16384 --k 17 --cands tma2,tma3 --scheds 0:0,9:148,18:148"""
+    python tools/sched_check.py --size 16384 --k 17 --cands tma2,tma3 --scheds 0:0,9:148,18:148,9:0:85
+(a schedule is parts:grid[:steal], steal = the tail-donation percent)"""
 import argparse
 import os
 import sys
@@ -17,6 +18,7 @@ ap.add_argument("--cands", default="tma2,tma3")
 ap.add_argument("--scheds", default="0:0,9:148,9:0,18:148,5:74")
 ap.add_argument("--n", type=int, default=10)
 ap.add_argument("--tune", action="store_true")
+ap.add_argument("--retime", action="store_true", help="with --tune: time the schedules again after tuning")
 a = ap.parse_args()
 H = W = a.size
 K = a.k
@@ -26,14 +28,10 @@ k = synth.binomial_kernel(K)
 p = sc.Plan(H, W, K)
 l2 = torch.cuda.get_device_properties(0).L2_cache_size
 cold = 8 * H * W <= 2 * l2
-wb = torch.empty(2 * l2 // 4, device="cuda")
-rb = torch.zeros(2 * l2 // 4, device="cuda")
-sink = torch.empty((), device="cuda")
 
 
 def flush():
-    wb.fill_(1.0)
-    torch.sum(rb, dim=0, out=sink)
+    sc.l2_flush()                                    # the bench's and the tuner's clean flush
 
 
 def batch(fn, n):
@@ -56,14 +54,22 @@ def t_pass(c):
     return sorted(ts)[1]
 
 
-for name in a.cands.split(","):
-    cfg = int(name.replace("tma", "").replace("s8", ""))
-    for sch in a.scheds.split(","):
-        parts, grid = (int(v) for v in sch.split(":"))
-        c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, 1 if name.endswith("s8") else 0, sched_parts=parts,
-                      sched_grid=grid)
-        print("%5d K=%2d %-14s parts %4d grid %4d: %8.2f us" % (H, K, c.base_name, parts, grid, t_pass(c)), flush=True)
+def sweep(tag=""):
+    for name in a.cands.split(","):
+        cfg = int(name.replace("tma", "").replace("s8", ""))
+        for sch in a.scheds.split(","):
+            v = [int(t) for t in sch.split(":")] + [0]
+            parts, grid, steal = v[0], v[1], v[2]
+            c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, 1 if name.endswith("s8") else 0,
+                          sched_parts=parts, sched_grid=grid, sched_steal=steal)
+            print("%5d K=%2d %-14s parts %4d grid %4d steal %2d: %8.2f us%s" % (H, K, c.base_name, parts, grid, steal,
+                                                                                 t_pass(c), tag), flush=True)
+
+
+sweep()
 if a.tune:
     for m in (-1, 12):
         b = p.tune(reps=10, force=True, mutations=m)
         print("tune(mutations=%d): %s %.2f us; re-timed %.2f us" % (m, b.name, b.median_us, t_pass(b)), flush=True)
+    if a.retime:
+        sweep("  (after tuning)")
