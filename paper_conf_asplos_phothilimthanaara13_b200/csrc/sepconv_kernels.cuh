@@ -182,9 +182,12 @@ struct OutCursor {
         ptr += ld;
     }
     // Fastest path: every row start is 16-byte aligned (out base, ld_out and image
-    // stride multiples of 4 floats): one predicated STG.128, nothing else.
+    // stride multiples of 4 floats): one predicated STG.128, nothing else.  `full` also
+    // admits the right-edge warp when the output width is a multiple of 4 (each lane's four
+    // columns are then all inside or all outside), so every warp of the pass runs this one
+    // loop body (see the dispatch in stream_kernel).
     __device__ __forceinline__ void store_fast16(const float (&v)[V], bool ok) {
-        const unsigned p16 = ok;
+        const unsigned p16 = ok && full;
         asm volatile(
             "{\n\t.reg .pred q16;\n\t"
             "setp.ne.u32 q16, %5, 0;\n\t"
@@ -674,7 +677,12 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         // (16-warp configurations take the 8-byte rows as two 8-byte stores: the shuffled form
         // spills at their 128-register budget)
         constexpr int SMF = (SM == 1 && NW >= 16) ? 3 : SM;
-        if (wcol + kWarpCols <= p.out_cols && p.store8 >= SM) run_chunks(std::integral_constant<int, SMF>{});
+        // The right-edge warp of a ragged width joins the 16-byte path when the width is a
+        // multiple of 4 (store_fast16 masks its outside lanes): a second copy of the ~38 KB
+        // K=17 loop running on some SMs slowed those CTAs and their TPC neighbours by 6-12%
+        // at 16384^2 (the last two CTA strips; profiles/r02_cta_strips.txt)
+        const bool fast = (wcol + kWarpCols <= p.out_cols || (SMF == 2 && (p.out_cols & 3) == 0)) && p.store8 >= SM;
+        if (fast) run_chunks(std::integral_constant<int, SMF>{});
         else run_chunks(std::integral_constant<int, 0>{});
     }
 #ifdef SEPCONV_CTA_TRACE

@@ -36,8 +36,8 @@ __global__ void read_k(const float4 *p, long long n, float *s) {
 }
 
 template <int K, int NW, int SR, int NS, int F2, int SM = 2, int LOCK = 0>
-static void trace_cfg(int H, const char *tag, int parts_mult = 1) {
-    const int W = H;
+static void trace_cfg(int H, const char *tag, int parts_mult = 1, int Win = 0) {
+    const int W = Win ? Win : H;
     auto kern = stream_kernel<K, OP_SEP, MAP_TMA, NW, SR, NS, F2, SM, LOCK>;
     const size_t smem = stream_smem_bytes<K, OP_SEP, MAP_TMA, NW, SR, NS, F2>();
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -51,7 +51,7 @@ static void trace_cfg(int H, const char *tag, int parts_mult = 1) {
     p.nstrips = (p.out_cols + NW * 128 - 1) / (NW * 128);
     p.total = (long long)p.nstrips * p.rows;
     for (int i = 0; i < K; ++i) { p.k[i] = 1.0f / K; p.k2[i] = make_float2(p.k[i], p.k[i]); }
-    p.store8 = 2;
+    p.store8 = ((W - K + 1) % 4 == 0) ? 2 : (((W - K + 1) % 2 == 0) ? 1 : 0);
     p.trace = dtrace;
     cuuint64_t dims[3] = {(cuuint64_t)W, (cuuint64_t)H, 1};
     cuuint64_t str[2] = {(cuuint64_t)W * 4, (cuuint64_t)H * W * 4};
@@ -96,17 +96,32 @@ static void trace_cfg(int H, const char *tag, int parts_mult = 1) {
         printf(" %d:%llu,%.1f,%llu", b, t[4 * b + 2], dur[b], t[4 * b + 3]);
     }
     printf("\n");
+    if (getenv("CTA_TRACE_STRIPS")) {                    // mean CTA duration per CTA strip
+        printf("    W=%d strips=%d by strip:", W, p.nstrips);
+        for (int q = 0; q < p.nstrips; ++q) {
+            double sum = 0;
+            int cnt = 0;
+            for (int b = q; b < grid; b += p.nstrips) sum += dur[b], ++cnt;
+            printf(" %.1f", cnt ? sum / cnt : 0.0);
+        }
+        printf("\n");
+    }
+    if (getenv("CTA_TRACE_DUMP")) {                      // per-SM duration, for stability checks
+        printf("    dump %s H=%d K=%d:", tag, H, K);
+        for (int b = 0; b < grid; ++b) printf(" %llu:%.2f", t[4 * b + 2], dur[b]);
+        printf("\n");
+    }
     fflush(stdout);
 }
 
-int main() {
+int main(int argc, char **argv) {
     void *fp = nullptr;
     cudaDriverEntryPointQueryResult q;
     cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fp, cudaEnableDefault, &q);
     enc = (EncodeTiledFn)fp;
     cudaDeviceProp prop;
     cudaGetDeviceProperties(&prop, 0);
-    const size_t big = (size_t)16384 * 16384 * 4;
+    const size_t big = (size_t)16384 * 17440 * 4;
     cudaMalloc(&din, big);
     cudaMalloc(&dout, big);
     cudaMemset(din, 0, big);
@@ -116,6 +131,20 @@ int main() {
     cudaMalloc(&sink, 16);
     cudaMalloc(&dtrace, 4 * 4096 * 8);
     cudaMemset(rfl, 0, fl_n4 * 16);
+    if (argc > 1 && !strcmp(argv[1], "strips")) {         // which strips are slow, and why
+        for (int W : {16384, 16400, 16128, 15376, 17424}) trace_cfg<17, 8, 17, 2, 2>(16384, "tma4", 1, W);
+        for (int W : {16384, 16400}) trace_cfg<9, 8, 9, 2, 1, 2, 1>(16384, "tma0", 1, W);
+        return 0;
+    }
+    if (argc > 1 && !strcmp(argv[1], "stability")) {      // the same launches repeated
+        for (int rep = 0; rep < 3; ++rep) {
+            trace_cfg<17, 8, 17, 2, 2>(16384, "tma4");
+            trace_cfg<17, 8, 17, 2, 1>(16384, "tma2");
+            trace_cfg<9, 8, 9, 2, 1, 2, 1>(16384, "tma0");
+            trace_cfg<17, 8, 17, 2, 2>(4096, "tma4");
+        }
+        return 0;
+    }
     for (int H : {2048, 4096, 16384}) {
         trace_cfg<17, 8, 17, 2, 2>(H, "tma4");
         trace_cfg<17, 8, 17, 2, 1>(H, "tma2");
