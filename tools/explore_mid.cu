@@ -140,6 +140,33 @@ int main(int argc, char **argv) {
     cudaEventCreate(&e1);
     // (EXPLORE_CS, CTA-shared stages: measured and rejected in round 2, the kernel code reverted;
     //  profiles/r02_explore_cta_stage.txt)
+    // (EXPLORE_IWARM, a dry pass over the hot loop before the first segment to pull its code into the
+    //  instruction caches while the prologue loads fly: 2-12% slower at 2048-4096^2, reverted;
+    //  profiles/r02_explore_iwarm.txt)
+    if (getenv("EXPLORE_DEEP")) {                  // deeper free-running rings for short segments
+        for (int H : sizes) {
+            run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
+            run_cfg<3, 8, 6, 9, 1, 1>(H, "8w9s");
+            run_cfg<3, 8, 6, 6, 1, 1>(H, "8w6s");
+            run_cfg<3, 8, 6, 4, 1, 1>(H, "8w4s");
+            run_cfg<3, 8, 6, 6, 1, 1, 1>(H, "8w6s-lock");
+            run_cfg<3, 4, 6, 4, 1, 1>(H, "4w4s-x2", 2);
+            run_cfg<5, 8, 5, 2, 1, 2>(H, "tma2");
+            run_cfg<5, 8, 5, 8, 1, 2>(H, "8w8s");
+            run_cfg<7, 8, 7, 2, 1, 1>(H, "tma2");
+            run_cfg<7, 8, 7, 6, 1, 1>(H, "8w6s");
+            run_cfg<7, 4, 7, 2, 1, 1>(H, "tma5", 2);
+            run_cfg<7, 4, 7, 4, 1, 1>(H, "4w4s-x2", 2);
+            run_cfg<9, 8, 9, 2, 1, 2>(H, "tma2");
+            run_cfg<9, 8, 9, 5, 1, 2>(H, "8w5s");
+            run_cfg<9, 4, 9, 2, 1, 2>(H, "tma5", 2);
+            run_cfg<11, 8, 11, 2, 1, 1>(H, "tma2");
+            run_cfg<11, 8, 11, 4, 1, 1>(H, "8w4s");
+            run_cfg<13, 8, 13, 2, 1, 2>(H, "tma2");
+            run_cfg<13, 8, 13, 3, 1, 2>(H, "8w3s");
+        }
+        return 0;
+    }
     if (getenv("EXPLORE_K17")) {                   // round-2 follow-up: packed-FP32 row pass variants at K=17
         for (int H : sizes) {
             run_cfg<17, 8, 17, 2, 2>(H, "rowffma2");
