@@ -136,6 +136,16 @@ int main(int argc, char **argv) {
         for (int W : {16384, 16400}) trace_cfg<9, 8, 9, 2, 1, 2, 1>(16384, "tma0", 1, W);
         return 0;
     }
+    if (argc > 1 && !strcmp(argv[1], "mid")) {            // mid sizes after the right-edge change
+        for (int rep = 0; rep < 2; ++rep)
+            for (int H : {2048, 4096}) {
+                trace_cfg<17, 8, 17, 2, 2>(H, "tma4");
+                trace_cfg<17, 8, 17, 2, 1>(H, "tma2");
+                trace_cfg<17, 16, 17, 1, 1>(H, "tma3");
+                trace_cfg<9, 8, 9, 2, 1, 2, 1>(H, "tma0");
+            }
+        return 0;
+    }
     if (argc > 1 && !strcmp(argv[1], "stability")) {      // the same launches repeated
         for (int rep = 0; rep < 3; ++rep) {
             trace_cfg<17, 8, 17, 2, 2>(16384, "tma4");
