@@ -143,6 +143,17 @@ int main(int argc, char **argv) {
     // (EXPLORE_IWARM, a dry pass over the hot loop before the first segment to pull its code into the
     //  instruction caches while the prologue loads fly: 2-12% slower at 2048-4096^2, reverted;
     //  profiles/r02_explore_iwarm.txt)
+    if (getenv("EXPLORE_HINT")) {                  // store cache hint (compile with -DSEPCONV_ST_HINT='".cs"')
+        for (int H : sizes) {
+            run_cfg<17, 8, 17, 2, 2>(H, "tma4");
+            run_cfg<17, 8, 17, 2, 1>(H, "tma2");
+            run_cfg<9, 8, 9, 2, 1, 2, 1>(H, "tma0");
+            run_cfg<9, 4, 9, 2, 1, 2>(H, "tma5", 2);
+            run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
+            run_cfg<5, 8, 5, 2, 1, 2>(H, "tma2");
+        }
+        return 0;
+    }
     if (getenv("EXPLORE_DEEP")) {                  // deeper free-running rings for short segments
         for (int H : sizes) {
             run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
