@@ -8,7 +8,7 @@ import numpy as np
 import pytest
 
 import oracle
-from paper_conf_asplos_phothilimthanaara13_b200 import sor, synth
+from paper_conf_asplos_phothilimthanaara13_b200 import sepconv as sc, sor, synth
 
 torch = pytest.importorskip("torch")
 pytestmark = pytest.mark.gpu
@@ -84,6 +84,61 @@ def test_iterates_bitwise_vs_f32_oracle(shape, variant, depth):
         got = gpu_solve(x, b, omega, iters, variant, depth)
         want = oracle.sor_rb_f32(x, b, omega, iters)
         assert np.array_equal(got, want), f"iters={iters}: max diff {np.max(np.abs(got - want))}"
+
+
+@pytest.mark.parametrize("variant,depth", [("half", 0), ("wave", 2), ("wave", 3)])
+def test_graph_replay_bitwise_and_counted(variant, depth):
+    """sor_iterate records a multi-launch call as a CUDA graph and replays it for the next call
+    with the same key (omega, iterations, variant, depth, schedule, starting buffer pair): the
+    replays -- from both buffer pairs -- stay bitwise equal to the oracle and count the launches
+    they execute."""
+    n, m = 257, 1031
+    x, b = synth.poisson_problem(n, m, seed=5, guess="uniform")
+    omega = synth.omega_opt(n, m)
+    p = sor.SorPlan(n, m)
+    if depth:
+        p.set_depth(depth)
+    dx, db = _dev(x), _dev(b)
+    u = torch.empty((n, m), device="cuda")
+    iters = 5
+    launches = 2 * iters if variant == "half" else -(-iters // depth)
+    want = {k: oracle.sor_rb_f32(x, b, omega, k * iters) for k in (1, 2)}
+    for rep in range(3):                  # rep 0 records, later reps replay
+        p.load(dx, db)
+        for k in (1, 2):                  # the second call starts where the first left the pair index
+            c0 = sc.launch_count()
+            p.iterate(omega, iters, variant)
+            torch.cuda.synchronize()
+            assert sc.launch_count() - c0 == launches
+            p.store(u)
+            torch.cuda.synchronize()
+            got = u.cpu().numpy()
+            assert np.array_equal(got, want[k]), f"rep {rep} call {k}: max diff {np.max(np.abs(got - want[k]))}"
+
+
+def test_graph_replay_inside_a_callers_capture():
+    """A caller capturing its own stream gets the direct launches (no nested capture): the
+    captured call replays bitwise equal to the oracle.  As with any stateful call under capture,
+    the plan's host-side state (which buffer pair holds the iterate) advances when the call is
+    captured, and the replay performs the recorded passes."""
+    n, m = 130, 300
+    x, b = synth.poisson_problem(n, m, seed=9, guess="uniform")
+    omega = 1.5
+    p = sor.SorPlan(n, m)
+    p.set_depth(2)
+    p.load(_dev(x), _dev(b))
+    torch.cuda.synchronize()
+    g = torch.cuda.CUDAGraph()
+    s = torch.cuda.Stream()
+    with torch.cuda.graph(g, stream=s):
+        p.iterate(omega, 6, "wave", torch.cuda.current_stream())
+    torch.cuda.synchronize()
+    g.replay()                            # the capture executed nothing; the replay runs the passes
+    torch.cuda.synchronize()
+    u = torch.empty((n, m), device="cuda")
+    p.store(u)
+    torch.cuda.synchronize()
+    assert np.array_equal(u.cpu().numpy(), oracle.sor_rb_f32(x, b, omega, 6))
 
 
 @pytest.mark.parametrize("omega", [0.7, 1.0, 1.5, 1.97])
