@@ -60,7 +60,12 @@ sepconv_status_t sor_load(sor_plan_t plan, const float *x, int64_t ld_x, const f
                           sepconv_stream_t stream);
 
 /* P3-P4: `iters` >= 0 red-black iterations with relaxation factor 0 < omega < 2 on
- * the split buffers.  E_INVALID for omega outside (0, 2) or iters < 0. */
+ * the split buffers.  E_INVALID for omega outside (0, 2) or iters < 0.
+ * A call of two or more kernel launches is recorded (on its first use) as a CUDA graph keyed by
+ * omega, iters, variant, depth, schedule and the buffer pair it starts from, and replayed on
+ * `stream` by later calls with the same key (env SOR_GRAPHS=0: always direct launches).  If
+ * `stream` is being captured by the caller, the launches go into the caller's capture; the
+ * plan's host-side state (which pair holds the iterate) advances at capture time. */
 sepconv_status_t sor_iterate(sor_plan_t plan, float omega, int iters, sor_variant_t variant,
                              sepconv_stream_t stream);
 
