@@ -480,6 +480,8 @@ def main():
     for K in widths:
         choices[K] = plans[K].tune(reps=args.tune_reps, mutations=args.tune_mutations)
     torch.cuda.synchronize()
+    l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
+    flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
 
     def one_pass(K):
         if world > 1 and args.workload == "image":
@@ -506,8 +508,6 @@ def main():
     # width the flushed mode times `steps` x [flush, pass] and `steps` x [flush] between event
     # pairs and takes the difference (time_flushed): the marginal device time of the pass inside
     # a stream of work, as the unflushed mode measures it.
-    l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
-    flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
     do_flush = CleanFlush(torch, dev) if flush else None
 
     def evpair():
@@ -677,7 +677,9 @@ def main():
               "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": cfg,
               "hbm_gbs": sum(alg_bytes(K) for K in widths) / (ms_per_step * 1e-3) / 1e9,
               "per_width": per_width, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
-              "gpu_launches": int(launches), "clocks": clk.summary()})
+              "gpu_launches": int(launches), "clocks": clk.summary(),
+              "tuning": f"sepconv_tune per width (reps {args.tune_reps}; flushed when the inputs fit in L2, else "
+                        "back to back)"})
     if dist:
         dist.barrier()
         dist.destroy_process_group()

@@ -848,4 +848,27 @@ sepconv_status_t sepconv_get_choice(sepconv_plan_t plan, sepconv_variant_t varia
     return SEPCONV_OK;
 }
 
+sepconv_status_t sepconv_set_choice(sepconv_plan_t plan, sepconv_variant_t variant, const sepconv_choice_t *choice) {
+    clear_error();
+    if (!plan) return fail(SEPCONV_E_INVALID, "plan is NULL");
+    if (variant != SEPCONV_2D && variant != SEPCONV_SEPARABLE && variant != SEPCONV_AUTO)
+        return fail(SEPCONV_E_INVALID, "bad variant");
+    sepconv_status_t s = check_choice(choice);
+    if (s != SEPCONV_OK) return s;
+    if (variant != SEPCONV_AUTO && choice->algo != static_cast<int>(variant))
+        return fail(SEPCONV_E_INVALID, "choice.algo does not belong to the variant it is set for");
+    if (!plan->tuned) {                                        // the others keep their resolution
+        for (int v = 0; v < 3; ++v) {
+            const sepconv_variant_t vv = v == 0 ? SEPCONV_2D : v == 1 ? SEPCONV_SEPARABLE : SEPCONV_AUTO;
+            plan->best[v] = to_choice(resolve(plan, vv), plan->k, SEPCONV_SRC_DEFAULT);
+        }
+        plan->tuned = true;
+    }
+    const int idx = variant == SEPCONV_2D ? 0 : variant == SEPCONV_SEPARABLE ? 1 : 2;
+    sepconv_choice_t c = to_choice(from_choice(*choice), plan->k, SEPCONV_SRC_EXPLICIT);
+    c.median_us = choice->median_us;
+    plan->best[idx] = c;
+    return SEPCONV_OK;
+}
+
 }  // extern "C"

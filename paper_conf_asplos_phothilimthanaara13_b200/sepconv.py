@@ -165,6 +165,7 @@ def lib() -> ctypes.CDLL:
                                           ctypes.POINTER(_Selector)]),
             "sepconv_select": (I, [ctypes.POINTER(_Selector), I64, ctypes.POINTER(_Choice)]),
             "sepconv_get_choice": (I, [P, I, ctypes.POINTER(_Choice)]),
+            "sepconv_set_choice": (I, [P, I, ctypes.POINTER(_Choice)]),
             "sepconv_num_candidates": (I, [P]),
             "sepconv_get_candidate": (I, [P, I, ctypes.POINTER(_Choice)]),
             "sepconv_band": (I, [I64, I, I, I, pI64, pI64, pI64, pI64]),
@@ -210,7 +211,7 @@ def launch_count() -> int:
 def exported_symbols():
     return ["sepconv_plan", "sepconv_plan_ex", "sepconv_destroy", "sepconv_out_shape", "sepconv_run",
             "sepconv_run_choice", "sepconv_run_host", "sepconv_tune", "sepconv_tune_selector", "sepconv_select",
-            "sepconv_get_choice",
+            "sepconv_get_choice", "sepconv_set_choice",
             "sepconv_num_candidates", "sepconv_get_candidate", "sepconv_band", "sepconv_nccl_unique_id",
             "sepconv_comm_init", "sepconv_run_band", "sepconv_band_trace", "sepconv_band_timeline",
             "sepconv_status_str", "sepconv_last_error",
@@ -357,6 +358,11 @@ class Plan:
         out = _Choice()
         _check(lib().sepconv_get_choice(self._h, _variant(variant), ctypes.byref(out)), "sepconv_get_choice")
         return Choice._from(out)
+
+    def set_choice(self, choice: Choice, variant="auto"):
+        """sepconv_set_choice: `variant` resolves to `choice` on this plan from now on."""
+        c = choice._c()
+        _check(lib().sepconv_set_choice(self._h, _variant(variant), ctypes.byref(c)), "sepconv_set_choice")
 
     def candidates(self):
         res = []

@@ -196,3 +196,14 @@ def test_choice_names_and_steal_field():
     assert sc.Choice._from(c._c()) == c
     assert sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 2, sched_steal=4).name == "sep-fused-tma2"
     assert [f[0] for f in sc._Choice._fields_][-2:] == ["sched_steal", "source"]
+
+
+def test_set_choice_validation_before_device():
+    """sepconv_set_choice rejects a NULL plan, a NULL choice and a malformed one without a device."""
+    import ctypes
+    L = sc.lib()
+    c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 0)._c()
+    assert L.sepconv_set_choice(None, 2, ctypes.byref(c)) == -1
+    bad = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 99)._c()
+    assert L.sepconv_set_choice(None, 2, ctypes.byref(bad)) == -1
+    assert L.sepconv_set_choice(None, 2, None) == -1

@@ -156,6 +156,30 @@ def test_variants_and_auto_default():
         check(img, k, run_gpu(img, k, variant=v)[0])
 
 
+def test_set_choice_drives_auto():
+    """sepconv_set_choice: AUTO resolves to the set candidate (bitwise the output run_choice gives
+    for it, within the bound of the oracle), the other variants keep their resolution, and a
+    choice of the wrong algorithm for a variant is rejected."""
+    h, w, K = 300, 1100, 7
+    img = synth.uniform_image(h, w, seed=77)
+    k = synth.binomial_kernel(K)
+    p = sc.Plan(h, w, K)
+    sep_before = p.get_choice("separable")
+    for cfg in (3, 5):
+        c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg)
+        p.set_choice(c)
+        got = p.get_choice("auto")
+        assert got.key() == c.key() and got.source == sc.SRC_EXPLICIT
+        assert p.get_choice("separable").key() == sep_before.key()
+        via_auto = run_gpu(img, k, variant="auto", plan=p)[0]
+        via_choice = run_gpu(img, k, c, plan=p)[0]
+        assert np.array_equal(via_auto, via_choice)
+        check(img, k, via_auto)
+    with pytest.raises(sc.SepconvError) as ei:
+        p.set_choice(sc.Choice(sc.SEPCONV_2D, sc.MAP_TMA, 0), "separable")
+    assert ei.value.code == "E_INVALID"
+
+
 def test_tune_choice_is_valid_and_cached(tmp_path):
     cache = str(tmp_path / "tune.jsonl")
     img = synth.uniform_image(512, 768, seed=9)
