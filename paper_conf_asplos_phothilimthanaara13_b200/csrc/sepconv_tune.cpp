@@ -391,7 +391,7 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
     // (fused TMA with free-running warps, at most 8 per CTA: cfg 2, 4, 5)
     const bool stealing = best.algo == SEPCONV_SEPARABLE && best.fused && best.mapping == SEPCONV_MAP_TMA &&
                           (best.config == 2 || best.config == 4 || best.config == 5);
-    const int nseeds = stealing ? 4 : 2;
+    const int nseeds = stealing ? 6 : 4;
     int steal = best.sched_steal;
     for (int m = 0; m < mutations + nseeds; ++m) {
         double np = parts, ng = grid;
@@ -403,10 +403,18 @@ sepconv_status_t mutate_schedule(Bench &b, Candidate &best, float &best_us, int 
             np = parts0 * (m + 2);
             ng = static_cast<double>(slots);
             nst = 0;
+        } else if (m < 4) {
+            // ... and 2/3 and 1/2 of one round on as many CTAs as items: fewer, taller segments
+            // on fewer SMs.  HBM-bound widths stream from fewer concurrent row windows
+            // (16384^2 / K=5: cfg 1 with 6 parts on 96 CTAs 328 us against 375 us under the model's
+            // schedule and 351 us for the best default, profiles/r02p_tune_diag.txt)
+            np = std::max(1.0, std::round(parts0 * (m == 2 ? 2.0 / 3.0 : 0.5)));
+            ng = std::min(static_cast<double>(slots), static_cast<double>(strips) * np);
+            nst = 0;
         } else if (m < nseeds) {
             // stealing on one and on two rounds of the model's items: warps that run out of
             // work take half of the largest unclaimed remainder (profiles/r02_steal_sched.txt)
-            np = parts0 * (m - 1);
+            np = parts0 * (m - 3);
             ng = static_cast<double>(slots);
             nst = 4;
         } else {
@@ -550,13 +558,32 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
         us[s] = med[bi[s]];
     }
     // the paper's evolutionary refinement of size-like tunables, on each single-kernel finalist
-    // (up to four): a configuration that loses under the model's schedule can win under its
+    // (up to six, below): a configuration that loses under the model's schedule can win under its
     // own best schedule (16384^2 / K=17: cfg 4 with 27 parts beats cfg 3, which gains nothing;
     // the fourth finalist is kept for configurations that only win with work stealing)
     if (mutations > 0) {
+        // the pool: the single-kernel finalists, then, for every other single-kernel mapping /
+        // configuration within 15% of the fastest under the model's schedule, its faster store
+        // path: a configuration 7% behind under the model's schedule was 7% ahead under its own
+        // (16384^2 / K=5, cfg 1: 375 -> 328 us with 6 parts on 96 CTAs, profiles/r02p_tune_diag.txt)
         std::vector<size_t> pool;
         for (size_t i : finalists)
             if (passes(cs[i]) == 1 && pool.size() < 4) pool.push_back(i);
+        {
+            const float fastest = *std::min_element(med.begin(), med.end());
+            auto same_kernel = [&](size_t a, size_t c) {
+                return cs[a].algo == cs[c].algo && cs[a].mapping == cs[c].mapping && cs[a].fused == cs[c].fused &&
+                       cs[a].config == cs[c].config;
+            };
+            std::vector<size_t> more;
+            for (size_t i = 0; i < cs.size(); ++i)
+                if (med[i] >= 0 && med[i] <= fastest * 1.15f && passes(cs[i]) == 1)
+                    more.push_back(i);
+            std::sort(more.begin(), more.end(), [&](size_t a, size_t c) { return med[a] < med[c]; });
+            for (size_t i : more)
+                if (std::none_of(pool.begin(), pool.end(), [&](size_t j) { return same_kernel(i, j); }))
+                    pool.push_back(i);
+        }
         if (pool.empty()) pool.push_back(bi[2]);
         std::vector<std::pair<Candidate, float>> out;
         for (size_t i : pool) {

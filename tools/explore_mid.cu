@@ -154,6 +154,27 @@ int main(int argc, char **argv) {
         }
         return 0;
     }
+    if (getenv("EXPLORE_DEEPLOCK")) {              // deeper lockstep rings for the HBM-bound small widths
+        for (int rep = 0; rep < 2; ++rep)
+            for (int H : sizes) {
+                run_cfg<3, 8, 6, 2, 1, 1, 1>(H, "tma0");
+                run_cfg<3, 8, 9, 3, 1, 1, 1>(H, "tma1");
+                run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
+                run_cfg<3, 8, 6, 4, 1, 1, 1>(H, "8w4s-lock");
+                run_cfg<3, 8, 6, 6, 1, 1, 1>(H, "8w6s-lock");
+                run_cfg<3, 8, 9, 5, 1, 1, 1>(H, "8w5sx9-lock");
+                run_cfg<5, 8, 5, 2, 1, 2, 1>(H, "tma0");
+                run_cfg<5, 8, 10, 3, 1, 2, 1>(H, "tma1");
+                run_cfg<5, 8, 5, 2, 1, 2>(H, "tma2");
+                run_cfg<5, 8, 5, 6, 1, 2, 1>(H, "8w6s-lock");
+                run_cfg<5, 8, 10, 5, 1, 2, 1>(H, "8w5sx10-lock");
+                run_cfg<7, 8, 7, 2, 1, 1, 1>(H, "tma0");
+                run_cfg<7, 8, 7, 2, 1, 1>(H, "tma2");
+                run_cfg<7, 8, 7, 5, 1, 1, 1>(H, "8w5s-lock");
+                run_cfg<7, 8, 14, 3, 1, 1, 1>(H, "8w3sx14-lock");
+            }
+        return 0;
+    }
     if (getenv("EXPLORE_DEEP")) {                  // deeper free-running rings for short segments
         for (int H : sizes) {
             run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
