@@ -18,20 +18,22 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--size", type=int, default=16384)
     ap.add_argument("--widths", default="3,5,7")
+    ap.add_argument("--batch", type=int, default=1, help="images per plan (BASELINE C5: 64 x 4096^2)")
     a = ap.parse_args()
     dev = torch.device("cuda", 0)
     H = W = a.size
     st = torch.cuda.current_stream(dev)
-    img = torch.from_numpy(synth.uniform_image(H, W, synth.BENCH_SEED_BASE + 3)).to(dev)
+    img = torch.rand((a.batch, H, W), device=dev)
     for K in [int(x) for x in a.widths.split(",")]:
-        p = sc.Plan(H, W, K)
-        out = torch.empty((H - K + 1, W - K + 1), device=dev)
+        p = sc.Plan(H, W, K, n=a.batch)
+        out = torch.empty((a.batch, H - K + 1, W - K + 1), device=dev)
         k = synth.binomial_kernel(K)
         pick = p.tune(reps=10)
         print(f"K={K} tuner pick {pick.name} {pick.median_us:.1f} us", flush=True)
         trials = [pick]
         for cfg in range(6):
-            for parts, grid in ((0, 0), (6, 96), (9, 144), (18, 148), (27, 148)):
+            for parts, grid in (((0, 0), (6, 96), (9, 144), (18, 148), (27, 148)) if a.batch == 1 else
+                                ((0, 0), (1, 96), (1, 120), (1, 132), (1, 148), (2, 148))):
                 trials.append(sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, 0, sched_parts=parts, sched_grid=grid))
         res = []
         for rnd in range(2):
