@@ -572,10 +572,13 @@ def main():
                              "frac_of_measured": gbs / (peak_gbs * world),
                              "frac_of_8tbs": gbs / (NOMINAL_HBM_GBS * world)}
 
-    # roofline for the dominant kernel family (the AUTO choice of most widths)
-    names = [per_width[str(K)]["variant"] for K in widths]
-    dom = max(set(names), key=lambda n: sum(per_k_ms[K] for K in widths if per_width[str(K)]["variant"] == n))
-    dom_k = [K for K in widths if per_width[str(K)]["variant"] == dom]
+    # roofline for the dominant kernel (the compiled candidate with the largest share of the step;
+    # a tuned work-schedule override "@p..g.." is a launch parameter of the same kernel)
+    def kname(K):
+        return per_width[str(K)]["variant"].split("@")[0]
+    names = [kname(K) for K in widths]
+    dom = max(set(names), key=lambda n: sum(per_k_ms[K] for K in widths if kname(K) == n))
+    dom_k = [K for K in widths if kname(K) == dom]
     dom_bytes = sum(alg_bytes(K) for K in dom_k) / world          # per GPU, per launch set
     dom_s = sum(per_k_ms[K] for K in dom_k) * 1e-3
     achieved = dom_bytes / dom_s / 1e9
@@ -584,7 +587,7 @@ def main():
     if os.path.exists(tr_path):
         try:
             tr = json.load(open(tr_path))
-            base = dom.split("@")[0]                       # ncu traffic is per candidate, any schedule
+            base = dom                                     # ncu traffic is per candidate, any schedule
             vals = [tr[f"{base}:K{K}"] for K in dom_k if f"{base}:K{K}" in tr and args.workload == "image"
                     and world == 1 and H == 16384]
             if len(vals) == len(dom_k):

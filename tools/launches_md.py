@@ -33,7 +33,7 @@ out.append("")
 line = "Total %.1f us for %d steps under ncu (%.1f us/step)" % (total, steps, total / steps)
 if a.bench:
     d = json.load(open(a.bench))
-    line += " vs %.0f us/step event-timed in `%s`" % (d["ms_per_step"] * 1e3, a.bench)
+    line += " (the same command printed %.0f us/step event-timed under ncu's serialised replay: not a bench value; `%s`)" % (d["ms_per_step"] * 1e3, a.bench)
 out.append(line + ".")
 open(a.out, "w").write("\n".join(out) + "\n")
 print("\n".join(out[-3:]))

@@ -32,7 +32,7 @@ def main():
         print(f"K={K} tuner pick {pick.name} {pick.median_us:.1f} us", flush=True)
         trials = [pick]
         for cfg in range(6):
-            for parts, grid in (((0, 0), (6, 96), (9, 144), (18, 148), (27, 148)) if a.batch == 1 else
+            for parts, grid in (((0, 0), (6, 96), (9, 144), (9, 148), (18, 148), (27, 148)) if a.batch == 1 else
                                 ((0, 0), (1, 96), (1, 120), (1, 132), (1, 148), (2, 148))):
                 trials.append(sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, 0, sched_parts=parts, sched_grid=grid))
         res = []
