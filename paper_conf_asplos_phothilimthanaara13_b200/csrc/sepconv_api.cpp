@@ -339,7 +339,11 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     const int map = tma ? 2 + std::min(std::max(cfg, 0), ntma - 1) : (vec ? 1 : 0);
     const int store8 = (aligned(out, 16) && (ld_out % 4) == 0 && (out_img % 4) == 0) ? 2
                        : (aligned(out, 8) && (ld_out % 2) == 0 && (out_img % 2) == 0) ? 1 : 0;
-    const int smode = (store8 == 2 && store_path == 0) ? 2 : 1;
+    // store mode 3 (8-byte rows, even-width right-edge warps on the fast path, K >= 13 fused
+    // TMA only): on images up to 8192 columns the edge warp's second loop copy costs 4-19%, on
+    // wider ones the extra per-row predicates cost more than it (profiles/r02x_edge8_ab.txt)
+    const int smode = (store8 == 2 && store_path == 0) ? 2
+                      : (op == OP_SEP && tma && K >= 13 && (out_cols % 2) == 0 && out_cols <= 8192) ? 3 : 1;
     KernelInfo ki = stream_info(op, map, K, smode);
     int occ = 0;
     sepconv_status_t s = prepare_func(ki, plan->dev.device, plan->dev, &occ);

@@ -143,71 +143,42 @@ struct OutCursor {
     long long ld;            // row pitch (floats)
     bool full;               // all 4 columns of this thread are inside the image
     bool e1, e2, e3, e0;     // column c+e is inside the image
-    bool last4;              // this thread's 4 columns end the row exactly
     __device__ __forceinline__ void init(float *rowp, long long ld_, int c, int out_cols) {
         ptr = rowp + c;
         ld = ld_;
         full = c + V <= out_cols;
-        last4 = c + V == out_cols;
         e0 = c < out_cols;
         e1 = c + 1 < out_cols;
         e2 = c + 2 < out_cols;
         e3 = c + 3 < out_cols;
     }
-    // Fast path: every row start is 8-byte aligned (checked by the host).  A 16-byte aligned row
-    // is one STG.128 per lane.  An 8-byte aligned row is re-cut into 16-byte aligned chunks with
-    // two shuffles -- lane l stores (lane l-1's v2, v3, its own v0, v1) -- plus one 8-byte store
-    // at each end of the warp's span, so every sector is written once and whole instead of twice
-    // in halves.  EDGE: the warp may be a right-edge warp of an even output width (each lane has
-    // 4, 2 or 0 columns inside): a lane with 2 stores 8 bytes, the last lane with 4 closes the
-    // span; the extra predicates cost a few instructions per row, so only the widths whose hot
-    // loop is large enough for a second copy of it to hurt (K >= 13) compile them
-    template <bool EDGE>
+    // Fast path: the warp's 128 columns are inside the image and every row start is
+    // 8-byte aligned (checked by the host).  A 16-byte aligned row is one STG.128 per
+    // lane.  An 8-byte aligned row is re-cut into 16-byte aligned chunks with two
+    // shuffles -- lane l stores (lane l-1's v2, v3, its own v0, v1) -- plus one 8-byte
+    // store at each end of the warp's 512-byte span, so every sector is written once
+    // and whole instead of twice in halves.
     __device__ __forceinline__ void store_fast(const float (&v)[V], bool ok, int lane) {
         const unsigned a8 = static_cast<unsigned>(reinterpret_cast<uintptr_t>(ptr)) & 8u;
         const float u2 = __shfl_up_sync(0xffffffffu, v[2], 1);
         const float u3 = __shfl_up_sync(0xffffffffu, v[3], 1);
-        if constexpr (EDGE) {
-            const bool in2 = e1;                               // columns c, c+1 inside
-            const unsigned p16 = ok && a8 == 0 && full;
-            const unsigned ph = ok && a8 == 0 && !full && in2;
-            const unsigned pm = ok && a8 != 0 && lane != 0 && in2;
-            const unsigned p0 = ok && a8 != 0 && lane == 0 && in2;
-            const unsigned p31 = ok && a8 != 0 && full && (lane == 31 || last4);
-            asm volatile(
-                "{\n\t.reg .pred q16, qh, qm, q0, q31;\n\t"
-                "setp.ne.u32 q16, %7, 0;\n\t"
-                "setp.ne.u32 qm, %8, 0;\n\t"
-                "setp.ne.u32 q0, %9, 0;\n\t"
-                "setp.ne.u32 q31, %10, 0;\n\t"
-                "setp.ne.u32 qh, %11, 0;\n\t"
-                "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t"
-                "@qh st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
-                "@qm st.global" SEPCONV_ST_HINT ".v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
-                "@q0 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
-                "@q31 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
-                ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(u2), "f"(u3), "r"(p16), "r"(pm), "r"(p0),
-                "r"(p31), "r"(ph)
-                : "memory");
-        } else {
-            const unsigned p16 = ok && a8 == 0;
-            const unsigned pm = ok && a8 != 0 && lane != 0;
-            const unsigned p0 = ok && a8 != 0 && lane == 0;
-            const unsigned p31 = ok && a8 != 0 && lane == 31;
-            asm volatile(
-                "{\n\t.reg .pred q16, qm, q0, q31;\n\t"
-                "setp.ne.u32 q16, %7, 0;\n\t"
-                "setp.ne.u32 qm, %8, 0;\n\t"
-                "setp.ne.u32 q0, %9, 0;\n\t"
-                "setp.ne.u32 q31, %10, 0;\n\t"
-                "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t"
-                "@qm st.global" SEPCONV_ST_HINT ".v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
-                "@q0 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
-                "@q31 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
-                ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(u2), "f"(u3), "r"(p16), "r"(pm), "r"(p0),
-                "r"(p31)
-                : "memory");
-        }
+        const unsigned p16 = ok && a8 == 0;
+        const unsigned pm = ok && a8 != 0 && lane != 0;
+        const unsigned p0 = ok && a8 != 0 && lane == 0;
+        const unsigned p31 = ok && a8 != 0 && lane == 31;
+        asm volatile(
+            "{\n\t.reg .pred q16, qm, q0, q31;\n\t"
+            "setp.ne.u32 q16, %7, 0;\n\t"
+            "setp.ne.u32 qm, %8, 0;\n\t"
+            "setp.ne.u32 q0, %9, 0;\n\t"
+            "setp.ne.u32 q31, %10, 0;\n\t"
+            "@q16 st.global" SEPCONV_ST_HINT ".v4.f32 [%0], {%1, %2, %3, %4};\n\t"
+            "@qm st.global" SEPCONV_ST_HINT ".v4.f32 [%0+-8], {%5, %6, %1, %2};\n\t"
+            "@q0 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
+            "@q31 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(u2), "f"(u3), "r"(p16), "r"(pm), "r"(p0),
+            "r"(p31)
+            : "memory");
         ptr += ld;
     }
     // Fastest path: every row start is 16-byte aligned (out base, ld_out and image
@@ -246,27 +217,24 @@ struct OutCursor {
     }
     // 8-byte rows without shuffles: two predicated 8-byte stores per lane (each 32-byte sector
     // is written in two halves by the two instructions); fewer live registers than store_fast
-    // (EDGE: a right-edge warp of an even output width; each lane stores the pairs that are inside)
-    template <bool EDGE>
     __device__ __forceinline__ void store_v2x2(const float (&v)[V], bool ok) {
-        const unsigned qa = ok && (!EDGE || e1), qb = ok && (!EDGE || full);
+        const unsigned q = ok;
         asm volatile(
-            "{\n\t.reg .pred qa, qb;\n\t"
-            "setp.ne.u32 qa, %5, 0;\n\t"
-            "setp.ne.u32 qb, %6, 0;\n\t"
-            "@qa st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
-            "@qb st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
-            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(qa), "r"(qb)
+            "{\n\t.reg .pred q8;\n\t"
+            "setp.ne.u32 q8, %5, 0;\n\t"
+            "@q8 st.global" SEPCONV_ST_HINT ".v2.f32 [%0], {%1, %2};\n\t"
+            "@q8 st.global" SEPCONV_ST_HINT ".v2.f32 [%0+8], {%3, %4};\n\t}"
+            ::"l"(ptr), "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "r"(q)
             : "memory");
         ptr += ld;
     }
     // MODE 2: 16-byte rows, 1: 8-byte rows (shuffled into 16-byte chunks), 3: 8-byte rows as
     // two 8-byte stores, 0: ragged edge / 4-byte rows
-    template <int MODE, bool EDGE = false>
+    template <int MODE>
     __device__ __forceinline__ void put(const float (&v)[V], bool ok, int lane) {
         if constexpr (MODE == 2) store_fast16(v, ok);
-        else if constexpr (MODE == 1) store_fast<EDGE>(v, ok, lane);
-        else if constexpr (MODE == 3) store_v2x2<EDGE>(v, ok);
+        else if constexpr (MODE == 1) store_fast(v, ok, lane);
+        else if constexpr (MODE == 3) store_v2x2(v, ok);
         else store_scalar(v, ok);
     }
     // write v to the cursor row if ok, then move to the next row
@@ -520,10 +488,6 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     // work stealing between warps: free-running warps only (lockstep CTAs share barriers; the
     // 16-warp CTAs' 128-register budget has no room for the claim state)
     constexpr bool STEAL = TMA && RING && !LOCK && NW <= 8;
-    // SM = 3: the 8-byte store path with even-width right-edge warps on it too (the host picks it
-    // for K >= 13 on images up to 8192 columns; see the store-path dispatch below)
-    constexpr bool EDGE8 = SM == 3;
-    constexpr int SMS = SM == 3 ? 1 : SM;                      // the store path proper
     const bool steal_on = STEAL && p.steal > 0 && p.parts > 0;
     bool thief = false;
     int n, s, q0, nrows;
@@ -679,9 +643,9 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
                         }
                     }
                     const int q = t - (K - 1);                 // output row completed by this step
-                    oc.put<SMODE, EDGE8>(acc[(pr + 1) % K], static_cast<unsigned>(q) < static_cast<unsigned>(nrows), lane);
+                    oc.put<SMODE>(acc[(pr + 1) % K], static_cast<unsigned>(q) < static_cast<unsigned>(nrows), lane);
                 } else {
-                    oc.put<SMODE, EDGE8>(b, t < nrows, lane);
+                    oc.put<SMODE>(b, t < nrows, lane);
                 }
             }
             if constexpr (TMA) {
@@ -709,22 +673,15 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         }
         };
         // SM (a template parameter) is the store path of warps wholly inside the image; the
-        // host instantiates SM = 2 when every row start is 16-byte aligned, else SM = 1 (or 3)
+        // host instantiates SM = 2 when every row start is 16-byte aligned, else SM = 1
         // (16-warp configurations take the 8-byte rows as two 8-byte stores: the shuffled form
         // spills at their 128-register budget)
-        constexpr int SMF = (SMS == 1 && NW >= 16) ? 3 : SMS;
+        constexpr int SMF = (SM == 1 && NW >= 16) ? 3 : SM;
         // The right-edge warp of a ragged width joins the 16-byte path when the width is a
         // multiple of 4 (store_fast16 masks its outside lanes): a second copy of the ~38 KB
         // K=17 loop running on some SMs slowed those CTAs and their TPC neighbours by 6-12%
         // at 16384^2 (the last two CTA strips; profiles/r02_cta_strips.txt)
-        // The same holds for the 8-byte store paths (SM = 3) when the output width is even: each
-        // lane then has 4, 2 or 0 columns inside and store_fast<EDGE8> / store_v2x2<EDGE8>
-        // predicate the pairs.  Measured (profiles/r02x_edge8_ab.txt): 2048^2 / K = 13-17
-        // -11-19%, 3520^2 -4-9%, but +2-6% at 16384^2 (the predicates cost every warp a few
-        // instructions per row, and there the edge warp is 1 of 128), and up to +10% for K = 7 at
-        // mid sizes -- hence the host's choice of SM = 3 only for K >= 13 and widths <= 8192
-        const bool edge_ok = SMF == 2 ? (p.out_cols & 3) == 0 : (EDGE8 && (p.out_cols & 1) == 0);
-        const bool fast = (wcol + kWarpCols <= p.out_cols || edge_ok) && p.store8 >= SMS;
+        const bool fast = (wcol + kWarpCols <= p.out_cols || (SMF == 2 && (p.out_cols & 3) == 0)) && p.store8 >= SM;
         if (fast) run_chunks(std::integral_constant<int, SMF>{});
         else run_chunks(std::integral_constant<int, 0>{});
     }

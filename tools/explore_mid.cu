@@ -154,6 +154,18 @@ int main(int argc, char **argv) {
         }
         return 0;
     }
+    if (getenv("EXPLORE_EDGE8")) {                 // 8-byte store paths with an even-width right edge
+        for (int H : sizes) {
+            run_cfg<15, 8, 15, 2, 1, 1>(H, "tma2");
+            run_cfg<15, 8, 15, 2, 1, 1, 1>(H, "tma0");
+            run_cfg<17, 8, 17, 2, 1, 1>(H, "tma2s8");
+            run_cfg<17, 8, 17, 2, 2, 1>(H, "tma4s8");
+            run_cfg<13, 8, 13, 3, 1, 1, 1>(H, "tma1s8");
+            run_cfg<11, 8, 11, 3, 1, 1, 1>(H, "tma1");
+            run_cfg<7, 8, 7, 2, 1, 1>(H, "tma2");
+        }
+        return 0;
+    }
     if (getenv("EXPLORE_DEEPLOCK")) {              // deeper lockstep rings for the HBM-bound small widths
         for (int rep = 0; rep < 2; ++rep)
             for (int H : sizes) {
