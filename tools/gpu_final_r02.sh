@@ -3,7 +3,7 @@
 # the Fig. 2 sweep, the ncu launch list of bench.py's timed region and two full captures.
 cd "${GRAFT_REPO_ROOT:-$(dirname "$0")/..}"
 mkdir -p gpurun_out
-R=r02z
+R=${ROUND:-r02z}
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.limit --format=csv > gpurun_out/${R}_nvsmi.txt 2>&1
 timeout -s KILL 1500 python -m pytest tests -x -q -m gpu > gpurun_out/${R}_pytest_gpu.log 2>&1; echo "pytest rc=$?" >> gpurun_out/${R}_pytest_gpu.log
 timeout -s KILL 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/${R}_smoke.log 2>&1; echo "smoke rc=$?" >> gpurun_out/${R}_smoke.log
