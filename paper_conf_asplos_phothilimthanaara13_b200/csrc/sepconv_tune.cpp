@@ -532,8 +532,14 @@ sepconv_status_t tune_plan(sepconv_plan_t plan, int reps, int flags, int mutatio
     // FMA-heaviest: 80% FMA-pipe active) loses up to 5% to the power cap (16384^2 / K=17: 372.6 us
     // in the tuner, 393 us in bench.py, profiles/r02_driver_bench.json).  Without a flush it is
     // charged 4% when compared; flushed (mid-size) passes keep their measured time.
+    // The same holds for the three-stage lockstep configuration (cfg 1) from K = 7 up: 330 us in
+    // the tuner, 348-398 us in bench.py at 16384^2 / K=7 (6 runs on 3 boxes), 329-335 vs 361-381 us
+    // at K=13, where the free-running cfg 2 moves 1-2% (profiles/r02zz_bench_c4.json,
+    // profiles/r02_sustained_confirm_rejected/); below K=7 (cfg 1 on 96 CTAs, 330-345 us in the
+    // bench) it keeps its measured time.
     auto eff = [&](const Candidate &c, float t) {
-        const bool heavy = c.algo == SEPCONV_SEPARABLE && c.fused && c.mapping == SEPCONV_MAP_TMA && c.config == 4;
+        const bool fused_tma = c.algo == SEPCONV_SEPARABLE && c.fused && c.mapping == SEPCONV_MAP_TMA;
+        const bool heavy = fused_tma && (c.config == 4 || (c.config == 1 && b.g.K >= 7));
         return (heavy && !b.need_flush) ? t * 1.04f : t;
     };
     auto better = [&](size_t a, size_t c) {   // is candidate a better than incumbent c?
