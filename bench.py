@@ -480,6 +480,19 @@ def main():
     for K in widths:
         choices[K] = plans[K].tune(reps=args.tune_reps, mutations=args.tune_mutations)
     torch.cuda.synchronize()
+    if world > 1:
+        # every rank runs rank 0's pick (sepconv_set_choice): the step ends with the slowest rank,
+        # and per-rank picks made under tuning noise would let the worst of them set the pace
+        for K in widths:
+            c = choices[K]
+            t = torch.tensor([c.algo, c.mapping, c.fused, c.config, c.store_path, c.sched_parts, c.sched_grid,
+                              c.sched_steal], dtype=torch.int64, device=dev)
+            dist.broadcast(t, 0)
+            if rank != 0:
+                v = [int(x) for x in t.tolist()]
+                plans[K].set_choice(sc.Choice(v[0], v[1], v[2], v[3], v[4], sched_parts=v[5], sched_grid=v[6],
+                                              sched_steal=v[7]))
+                choices[K] = plans[K].get_choice("auto")
     l2_bytes = torch.cuda.get_device_properties(dev).L2_cache_size or 126 * 2 ** 20
     flush = max(8 * (H * W * N_img) // max(world, 1), 0) <= 2 * l2_bytes
 
