@@ -156,6 +156,25 @@ def test_variants_and_auto_default():
         check(img, k, run_gpu(img, k, variant=v)[0])
 
 
+@pytest.mark.parametrize("cfg", range(6))
+@pytest.mark.parametrize("store_path", [0, 1])
+def test_right_edge_store_paths(cfg, store_path):
+    """Right-edge warps on the 8-byte store paths (store mode 3: fused TMA kernels, K >= 13,
+    widths <= 8192, even output widths): output widths = 2 and 0 mod 4, rows
+    8- and 16-byte aligned (a pitched output shifts every row start by 8 bytes), strips that end
+    inside a warp, next to the odd widths that keep the general store path -- every cell against
+    the oracle, canaries around every output."""
+    c = sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, cfg, store_path)
+    for w in (130, 642, 2048, 2051, 3520):
+        img = synth.uniform_image(40, w, seed=w) - np.float32(0.5)
+        for K in (13, 14, 15, 17):
+            k = synth.random_kernel(K, seed=K + w, signed=True)
+            wo = w - K + 1
+            for ld_out in (0, wo + 2, wo + 1):
+                out = run_gpu(img, k, c, ld_out=ld_out)[0]
+                check(img, k, out)
+
+
 def test_set_choice_drives_auto():
     """sepconv_set_choice: AUTO resolves to the set candidate (bitwise the output run_choice gives
     for it, within the bound of the oracle), the other variants keep their resolution, and a
