@@ -342,7 +342,8 @@ static sepconv_status_t launch_stream_op(sepconv_plan_t plan, int op, const Geom
     // store mode 3 (8-byte rows, even-width right-edge warps on the fast path, K >= 13 fused
     // TMA only): on images up to 8192 columns the edge warp's second loop copy costs 4-19%, on
     // wider ones the extra per-row predicates cost more than it (profiles/r02x_edge8_ab.txt)
-    const int smode = (store8 == 2 && store_path == 0) ? 2
+    const int smode = (op == OP_SEP && tma && store_path == 2) ? 4
+                      : (store8 == 2 && store_path == 0) ? 2
                       : (op == OP_SEP && tma && K >= 13 && (out_cols % 2) == 0 && out_cols <= 8192) ? 3 : 1;
     KernelInfo ki = stream_info(op, map, K, smode);
     int occ = 0;
@@ -759,7 +760,7 @@ static sepconv_status_t check_choice(const sepconv_choice_t *c) {
         return fail(SEPCONV_E_INVALID, "choice.mapping must be DIRECT or TMA");
     if (c->config < 0 || c->config >= kSepTmaConfigs)
         return fail(SEPCONV_E_INVALID, "choice.config must be in [0, %d)", kSepTmaConfigs);
-    if (c->store_path < 0 || c->store_path > 1) return fail(SEPCONV_E_INVALID, "choice.store_path must be 0 or 1");
+    if (c->store_path < 0 || c->store_path > 2) return fail(SEPCONV_E_INVALID, "choice.store_path must be 0, 1 or 2");
     if (c->sched_parts < 0 || c->sched_grid < 0)
         return fail(SEPCONV_E_INVALID, "choice.sched_parts / sched_grid must be >= 0");
     if (c->sched_steal < 0 || c->sched_steal > 99) return fail(SEPCONV_E_INVALID, "choice.sched_steal must be in [0, 99]");

@@ -52,10 +52,10 @@ static const StreamEntry *table(int op, int variant) {
 
 KernelInfo stream_info(int op, int variant, int K, int smode) {
     const StreamEntry *t = table(op, variant);
-    return t[K - 1].info[smode == 2 ? 1 : smode == 3 ? 2 : 0]();
+    return t[K - 1].info[smode == 2 ? 1 : smode == 3 ? 2 : smode == 4 ? 3 : 0]();
 }
 cudaError_t stream_launch(int op, int variant, int K, int smode, const StreamParams &p, int grid, cudaStream_t st) {
     const StreamEntry *t = table(op, variant);
-    return t[K - 1].launch[smode == 2 ? 1 : smode == 3 ? 2 : 0](p, grid, st);
+    return t[K - 1].launch[smode == 2 ? 1 : smode == 3 ? 2 : smode == 4 ? 3 : 0](p, grid, st);
 }
 }  // namespace sepconv

@@ -21,11 +21,12 @@ struct KernelInfo {
 // streaming kernels: op = OP_ROWS / OP_COLS / OP_SEP; variant = 0 direct, 1 direct 16-byte,
 // 2.. TMA configurations (stream_geom in sepconv_params.h); smode = 2 if every output row is
 // 16-byte aligned (the 16-byte store path), else 1, or 3 (the 8-byte path with even-width
-// right-edge warps on it; a distinct kernel only for the fused kernel at K >= 13).
+// right-edge warps on it; a distinct kernel only for the fused kernel at K >= 13), or 4 (two
+// 8-byte stores per lane: store path 2 of the fused TMA configurations).
 // conv2d: map = MAP_DIRECT / _VEC / MAP_TMA.  K in [1, 17].
 struct StreamEntry {
-    KernelInfo (*info[3])();
-    cudaError_t (*launch[3])(const StreamParams &, int, cudaStream_t);
+    KernelInfo (*info[4])();
+    cudaError_t (*launch[4])(const StreamParams &, int, cudaStream_t);
 };
 KernelInfo stream_info(int op, int variant, int K, int smode);
 cudaError_t stream_launch(int op, int variant, int K, int smode, const StreamParams &p, int grid, cudaStream_t st);

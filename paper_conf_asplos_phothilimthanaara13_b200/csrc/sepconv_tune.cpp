@@ -55,6 +55,12 @@ std::vector<Candidate> candidates(sepconv_plan_t p) {
     const bool rows16 = (p->ld_out % 4) == 0;
     if (rows16)
         for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 1});
+    // with 8-byte (not 16-byte) aligned rows, two 8-byte stores per lane instead of the shuffled
+    // 16-byte chunks (store path 2; the 16-warp cfg 3 already stores that way): a smaller loop
+    // body, faster on mid-size images, slower on large ones (profiles/r02_explore_v2x2.txt)
+    else if ((p->ld_out % 2) == 0)
+        for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg)
+            if (cfg != 3) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 2});
     cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1, 0, 0});
     cs.push_back({SEPCONV_2D, SEPCONV_MAP_TMA, 0, 0, 0});
     cs.push_back({SEPCONV_2D, SEPCONV_MAP_DIRECT, 0, 0, 0});
@@ -101,7 +107,7 @@ const char *parse_choice_at(const char *p, sepconv_choice_t *c) {
                    &parts, &grid, &steal, &used) != 11 || used == 0)
             return nullptr;
     }
-    if (store < 0 || store > 1 || config < 0 || config >= kSepTmaConfigs || parts < 0 || grid < 0) return nullptr;
+    if (store < 0 || store > 2 || config < 0 || config >= kSepTmaConfigs || parts < 0 || grid < 0) return nullptr;
     if (steal < 0 || steal > 99) return nullptr;
     if ((algo != SEPCONV_2D && algo != SEPCONV_SEPARABLE) || (map != 0 && map != 1)) return nullptr;
     std::memset(c, 0, sizeof *c);

@@ -84,7 +84,7 @@ class Choice:
         a = "2d" if self.algo == SEPCONV_2D else ("sep-fused" if self.fused else "sep-unfused")
         m = ("-tma" if self.mapping == MAP_TMA else "-direct")
         if self.algo == SEPCONV_SEPARABLE and self.fused and self.mapping == MAP_TMA:
-            m += "%d" % self.config + ("s8" if self.store_path else "")
+            m += "%d" % self.config + ("", "s8", "v2")[self.store_path]
         return a + m
 
     @property

@@ -12,8 +12,8 @@ cudaError_t no_launch(const StreamParams &, int, cudaStream_t) { return cudaErro
 StreamEntry kStub[kMaxK];
 const StreamEntry *stub_table() {
     for (auto &e : kStub) {
-        e.info[0] = e.info[1] = e.info[2] = no_info;
-        e.launch[0] = e.launch[1] = e.launch[2] = no_launch;
+        e.info[0] = e.info[1] = e.info[2] = e.info[3] = no_info;
+        e.launch[0] = e.launch[1] = e.launch[2] = e.launch[3] = no_launch;
     }
     return kStub;
 }

@@ -28,6 +28,8 @@ CANDS = [
     sc.Choice(sc.SEPCONV_2D, sc.MAP_DIRECT, 0),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 0),
     sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_DIRECT, 0),
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 1, 2),   # store path 2 (two 8-byte stores per lane)
+    sc.Choice(sc.SEPCONV_SEPARABLE, sc.MAP_TMA, 1, 4, 2),
 ]
 IDS = [c.name for c in CANDS]
 GUARD = 4096          # floats of NaN canary on each side of every output buffer
@@ -157,7 +159,7 @@ def test_variants_and_auto_default():
 
 
 @pytest.mark.parametrize("cfg", range(6))
-@pytest.mark.parametrize("store_path", [0, 1])
+@pytest.mark.parametrize("store_path", [0, 1, 2])
 def test_right_edge_store_paths(cfg, store_path):
     """Right-edge warps on the 8-byte store paths (store mode 3: fused TMA kernels, K >= 13,
     widths <= 8192, even output widths): output widths = 2 and 0 mod 4, rows

@@ -22,6 +22,7 @@ names["sep-fused-tma"] = names["sep-fused-tma0"]
 for cfg in range(8):                       # every fused TMA configuration, both store paths
     names["sep-fused-tma%d" % cfg] = (1, 1, 1, cfg)
     names["sep-fused-tma%ds8" % cfg] = (1, 1, 1, cfg, 1)
+    names["sep-fused-tma%dv2" % cfg] = (1, 1, 1, cfg, 2)
 H = W = a.size
 x = torch.rand((H, W), device="cuda")
 out = torch.empty((H - a.k + 1, W - a.k + 1), device="cuda")
