@@ -522,12 +522,16 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
     constexpr bool STEAL = TMA && RING && !LOCK && NW <= 8;
     // SM = 3: the 8-byte store path with even-width right-edge warps on it too (the host picks it
     // for K >= 13 on images up to 8192 columns; see the store-path dispatch below)
-    constexpr bool EDGE8 = SM == 3;
-    constexpr int SMS = (SM == 3 || SM == 4) ? 1 : SM;         // the store path proper
+    // store path 2 (SM = 4) carries its right-edge warp from K = 13 up as mode 3 does: two
+    // predicated 8-byte stores per lane instead of a second copy of the loop (2048^2 / K=15 19.2 ->
+    // 14.3 us, 3520^2 / 4096^2 -10%; mixed below K = 13, profiles/r02_explore_v2edge.txt)
+    constexpr bool EDGE8 = SM == 3 || SM == 5 || (SM == 4 && K >= 13);
+    constexpr int SMS = (SM >= 3) ? 1 : SM;                    // the store path proper
     // SM = 4 (store path 2): 8-byte rows as two 8-byte stores per lane at any warp count -- no
     // shuffles, a smaller loop body; faster at 2048^2-3520^2 (K = 7-15: -4-14%), slower at 16384^2
     // (each 32-byte sector written in two halves: +3-13%), so a tuner candidate
-    // (tools/explore_mid.cu EXPLORE_V2X2, profiles/r02_explore_v2x2.txt)
+    // (tools/explore_mid.cu EXPLORE_V2X2, profiles/r02_explore_v2x2.txt).  SM = 5 (exploration
+    // only): store path 2 with even-width right-edge warps on it (store_v2x2<EDGE>)
     const bool steal_on = STEAL && p.steal > 0 && p.parts > 0;
     bool thief = false;
     int n, s, q0, nrows;
@@ -716,7 +720,7 @@ __global__ void __launch_bounds__(NW * 32, MAP == MAP_TMA ? 1 : 2) stream_kernel
         // host instantiates SM = 2 when every row start is 16-byte aligned, else SM = 1 (or 3)
         // (16-warp configurations take the 8-byte rows as two 8-byte stores: the shuffled form
         // spills at their 128-register budget)
-        constexpr int SMF = (SM == 4 || (SMS == 1 && NW >= 16)) ? 3 : SMS;
+        constexpr int SMF = (SM == 4 || SM == 5 || (SMS == 1 && NW >= 16)) ? 3 : SMS;
         // The right-edge warp of a ragged width joins the 16-byte path when the width is a
         // multiple of 4 (store_fast16 masks its outside lanes): a second copy of the ~38 KB
         // K=17 loop running on some SMs slowed those CTAs and their TPC neighbours by 6-12%

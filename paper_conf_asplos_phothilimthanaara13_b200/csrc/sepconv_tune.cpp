@@ -57,8 +57,10 @@ std::vector<Candidate> candidates(sepconv_plan_t p) {
         for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 1});
     // with 8-byte (not 16-byte) aligned rows, two 8-byte stores per lane instead of the shuffled
     // 16-byte chunks (store path 2; the 16-warp cfg 3 already stores that way): a smaller loop
-    // body, faster on mid-size images, slower on large ones (profiles/r02_explore_v2x2.txt)
-    else if ((p->ld_out % 2) == 0)
+    // body, faster on mid-size images; on outputs wider than 8192 columns the half-sector writes
+    // lose (16384^2: K=11 +13%, K=15 +2-5% in the bench; profiles/r02_explore_v2x2.txt,
+    // profiles/r02v3_bench_c4*.json), so it is offered up to that width
+    else if ((p->ld_out % 2) == 0 && p->wo <= 8192)
         for (int cfg = 0; cfg < kSepTmaConfigs; ++cfg)
             if (cfg != 3) cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_TMA, 1, cfg, 2});
     cs.push_back({SEPCONV_SEPARABLE, SEPCONV_MAP_DIRECT, 1, 0, 0});

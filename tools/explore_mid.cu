@@ -90,7 +90,7 @@ static void run_cfg(int H, const char *tag, int cps_want = 1) {
     for (int i = 0; i < K; ++i) { p.k[i] = 1.0f / K; p.k2[i] = make_float2(p.k[i], p.k[i]); }
     p.store8 = ((W - K + 1) % 4 == 0) ? 2 : (((W - K + 1) % 2 == 0) ? 1 : 0);
     if (SM == 2 && p.store8 != 2) { printf("skip SM2 (rows not 16-byte aligned)\n"); return; }
-    if ((SM == 1 || SM == 4) && p.store8 < 1) { printf("skip SM%d (rows not 8-byte aligned)\n", SM); return; }
+    if ((SM == 1 || SM >= 3) && p.store8 < 1) { printf("skip SM%d (rows not 8-byte aligned)\n", SM); return; }
     cuuint64_t dims[3] = {(cuuint64_t)W, (cuuint64_t)H, 1};
     cuuint64_t str[2] = {(cuuint64_t)W * 4, (cuuint64_t)H * W * 4};
     cuuint32_t box[3] = {(cuuint32_t)stream_bw(K, OP_SEP), (cuuint32_t)SR, 1}, es[3] = {1, 1, 1};
@@ -153,6 +153,22 @@ int main(int argc, char **argv) {
             run_cfg<3, 8, 6, 2, 1, 1>(H, "tma2");
             run_cfg<5, 8, 5, 2, 1, 2>(H, "tma2");
         }
+        return 0;
+    }
+    if (getenv("EXPLORE_V2EDGE")) {                // store path 2 with / without the right-edge warp on it
+        for (int rep = 0; rep < 3; ++rep)
+            for (int H : sizes) {
+                run_cfg<3, 8, 9, 3, 1, 4, 1>(H, "tma1v2");
+                run_cfg<3, 8, 9, 3, 1, 5, 1>(H, "tma1v2e");
+                run_cfg<7, 8, 7, 2, 1, 4>(H, "tma2v2");
+                run_cfg<7, 8, 7, 2, 1, 5>(H, "tma2v2e");
+                run_cfg<7, 4, 7, 2, 1, 4>(H, "tma5v2", 2);
+                run_cfg<7, 4, 7, 2, 1, 5>(H, "tma5v2e", 2);
+                run_cfg<11, 8, 11, 2, 1, 4>(H, "tma2v2");
+                run_cfg<11, 8, 11, 2, 1, 5>(H, "tma2v2e");
+                run_cfg<15, 8, 15, 2, 1, 4>(H, "tma2v2");
+                run_cfg<15, 8, 15, 2, 1, 5>(H, "tma2v2e");
+            }
         return 0;
     }
     if (getenv("EXPLORE_V2X2")) {                  // 8-byte rows: shuffled 16-byte chunks (SM 1) vs two 8-byte stores (SM 4)
